@@ -1,0 +1,167 @@
+/*
+ * ppr.h -- C ABI of libppr.so: batch-parallel maintenance of Personalized
+ * PageRank (PPR) on a dynamic graph, on one NVIDIA B200 (sm_100a).
+ *
+ * The operation is the paper's problem statement (Guo, Li, Sha, Tan,
+ * "Parallel Personalized PageRank on Dynamic Graphs", PVLDB 11(1) 2017;
+ * cites "P:L" are lines of its text, PAPER.md):
+ *   - an initial graph G0 and a sequence of update sets E_t of arcs
+ *     (u, v, op), op in {insert, delete}
+ *   - for each unit-vector source s, maintain an estimate P_s and a residual
+ *     R_s satisfying the invariant (Eq. 2)
+ *        P(v) + a R(v) = (1-a)/d(v) * sum_{x in N_out(v)} P(x) + a 1[v=s]
+ *     and |R(v)| <= eps for all v, so |pi_s(v) - P(v)| <= eps.
+ *   - per batch: restore the invariant for all k updates (Alg 1, P:185-196,
+ *     in the batch closed form of Lemma 3's proof), then one
+ *     two-phase (POS, NEG) parallel local push (Alg 3 P:454-480 / Alg 4
+ *     P:1132-1157).
+ *   - pi_s is read as the reverse-PPR fixed point a (I-(1-a) D^-1 A)^-1 e_s
+ *     (reading R1; Eq. 1's W is Lemma 1's W^T = D^-1 A).
+ *
+ * Conventions for every call ("Boundary"):
+ *   - Every call returns ppr_status; PPR_OK == 0.
+ *   - Ownership: the caller owns every input array; it is consumed before
+ *     the call returns and no pointer is retained.  The library owns all
+ *     device state.  Output buffers are caller-allocated.
+ *   - Memory kinds: `mem` = PPR_MEM_HOST for host pointers (pageable or
+ *     pinned), PPR_MEM_DEVICE for device pointers on the handle's device,
+ *     valid in stream order on the handle's stream.
+ *   - Synchrony: calls return after the result is complete (the handle's
+ *     stream is synchronised).
+ *   - Validation happens before any mutation.  On PPR_EINVAL, PPR_ERANGE or
+ *     PPR_ENOENT the state is unchanged.  A CUDA failure returns PPR_ECUDA
+ *     and poisons the handle: every later call returns PPR_EPOISONED.
+ *   - Semantics: arcs form a multiset (a duplicate insertion raises the
+ *     multiplicity, Eq. 2 counts it); self-loops are allowed; the vertex set
+ *     is fixed to [0, n) (a vertex with no arcs is "absent");
+ *     within a batch insertions apply before deletions; an empty batch is a
+ *     no-op.  Vertex ids are uint32_t < n.
+ *   - Threading: a handle is bound to one device and is not thread-safe.
+ */
+#ifndef PPR_H
+#define PPR_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct ppr_ctx ppr_ctx; /* opaque; owned by the library */
+
+typedef enum {
+    PPR_OK = 0,
+    PPR_EINVAL = -1,    /* bad alpha / eps / n / sources / flags / option */
+    PPR_ERANGE = -2,    /* a vertex id >= n */
+    PPR_ENOENT = -3,    /* deletion of an arc absent after this batch's insertions */
+    PPR_ENOMEM = -4,    /* device or host allocation failed (state unchanged) */
+    PPR_ECUDA = -5,     /* CUDA error: the handle is poisoned */
+    PPR_EPOISONED = -6, /* an earlier call poisoned the handle */
+    PPR_ENOCONV = -7    /* push exceeded the iteration cap (handle poisoned) */
+} ppr_status;
+
+enum { PPR_MEM_HOST = 0, PPR_MEM_DEVICE = 1 };
+
+/* Parallel push variants of Table 3. */
+enum {
+    PPR_MODE_OPT = 0,       /* eager propagation + local duplicate detection (Alg 4);
+                               self-update fused with propagation (DESIGN.md K-PUSH) */
+    PPR_MODE_EAGER = 1,     /* eager propagation, UniqueEnqueue via bitmap */
+    PPR_MODE_DUPDETECT = 2, /* Alg 3 sessions + local duplicate detection */
+    PPR_MODE_VANILLA = 3    /* Alg 3 as printed: snapshot, barrier, propagate, UniqueEnqueue */
+};
+
+/* Graph for ppr_create: m arcs src[i] -> dst[i] on [0, n) (host pointers).
+ * undirected = 1 expands each {src,dst} into two arcs (one for a self-loop),
+ * P:868-870. */
+typedef struct {
+    uint32_t n;
+    uint64_t m;
+    const uint32_t *src;
+    const uint32_t *dst;
+    int undirected;
+} ppr_graph;
+
+/* Options for ppr_create; pass NULL for defaults. */
+typedef struct {
+    int device;          /* CUDA device ordinal (default 0) */
+    void *cuda_stream;   /* cudaStream_t to run on; NULL: the library creates one */
+    int mode;            /* PPR_MODE_* (default PPR_MODE_OPT) */
+    double slack;        /* slab slack fraction (default 0.25) */
+    uint32_t min_cap;    /* minimum slab capacity (default 4) */
+} ppr_opts;
+
+/* Per-call statistics (filled by ppr_create, ppr_apply_batch, ppr_push). */
+typedef struct {
+    uint32_t iters_pos, iters_neg;  /* frontier rounds per phase */
+    uint64_t pushes;                /* frontier vertices pushed (self-updates) */
+    uint64_t pushed_edges;          /* neighbour propagations (atomic adds) */
+    uint64_t max_frontier;          /* largest frontier seen */
+    uint64_t touched;               /* distinct (u, source) restored this batch */
+    uint64_t num_arcs;              /* arcs in the store after the call */
+    uint32_t rebuilt;               /* 1 if the slab store was rebuilt */
+    uint32_t kernel_launches;       /* kernels launched by this call */
+    float ms_total;                 /* CUDA-event time of the call on the stream */
+    float ms_store, ms_restore, ms_push; /* per phase (0 if timing disabled) */
+} ppr_batch_stats;
+
+/* Creates a handle: builds the slab store for g, sets P_s = 0 and R_s = e_s
+ * for every source (Eq. 2 holds trivially, Fig. 3 a(1)) and runs
+ * the two-phase push to convergence (static PPR).
+ * sources: num_sources distinct vertex ids < n (host pointer).
+ * 0 < alpha < 1, eps > 0 finite.  stats may be NULL. */
+ppr_status ppr_create(const ppr_graph *g, const uint32_t *sources, uint32_t num_sources,
+                      double alpha, double eps, const ppr_opts *opts, ppr_ctx **out,
+                      ppr_batch_stats *stats);
+
+/* Applies one batch: n_ins insertions ins_src[i] -> ins_dst[i] and n_del
+ * deletions del_src[i] -> del_dst[i] (arcs; undirected handles expand them),
+ * restores the invariant at every touched vertex for every source, then runs
+ * the two-phase push until |R| <= eps everywhere.  mem: PPR_MEM_HOST or
+ * PPR_MEM_DEVICE for the four input arrays.  stats may be NULL. */
+ppr_status ppr_apply_batch(ppr_ctx *h, const uint32_t *ins_src, const uint32_t *ins_dst,
+                           uint64_t n_ins, const uint32_t *del_src, const uint32_t *del_dst,
+                           uint64_t n_del, int mem, ppr_batch_stats *stats);
+
+/* Runs the two-phase push from a full scan of V (Alg 3 lines 1 and 4).
+ * Used after ppr_apply_batch with PPR_OPT_PUSH = 0.  stats may be NULL. */
+ppr_status ppr_push(ppr_ctx *h, ppr_batch_stats *stats);
+
+/* Resets every source to P_s = 0, R_s = e_s, which satisfies Eq. 2 for any
+ * graph (Fig. 3 a(1)); the next ppr_push recomputes static PPR. */
+ppr_status ppr_reset(ppr_ctx *h);
+
+/* Copies P_s (and R_s if R_out != NULL) of source number source_idx (its
+ * position in ppr_create's `sources`) into caller buffers of n doubles. */
+ppr_status ppr_query(ppr_ctx *h, uint32_t source_idx, double *P_out, double *R_out, int mem);
+
+/* Writes the arc multiset, sorted by (dst, src), into host buffers of `cap`
+ * entries; *m_out = number of arcs (PPR_EINVAL if cap is too small, with
+ * *m_out set). */
+ppr_status ppr_export_edges(ppr_ctx *h, uint32_t *src_out, uint32_t *dst_out, uint64_t cap,
+                            uint64_t *m_out);
+
+/* Copies d_out (n uint32_t) into a host buffer. */
+ppr_status ppr_export_dout(ppr_ctx *h, uint32_t *dout_out);
+
+/* Runtime options. */
+enum {
+    PPR_OPT_MODE = 1,      /* PPR_MODE_* for later pushes */
+    PPR_OPT_PUSH = 2,      /* 0: ppr_apply_batch stops after restore (tests); default 1 */
+    PPR_OPT_MAX_ITERS = 3, /* stop each phase after this many rounds (0 = run to eps) */
+    PPR_OPT_TIMING = 4,    /* 1: record per-phase CUDA events (default 1) */
+    PPR_OPT_FORCE_REBUILD = 5 /* 1: every batch takes the sort/merge rebuild path */
+};
+ppr_status ppr_set_option(ppr_ctx *h, int key, int64_t value);
+
+/* Device memory held by the handle, in bytes. */
+uint64_t ppr_device_bytes(const ppr_ctx *h);
+
+ppr_status ppr_destroy(ppr_ctx *h);
+const char *ppr_status_str(ppr_status s);
+const char *ppr_last_error(const ppr_ctx *h);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* PPR_H */

@@ -1,0 +1,735 @@
+// ppr_api.cu -- the C ABI of libppr.so (include/ppr.h) and the host
+// orchestrator of one batch:
+//
+//   a0 staging      H2D copy of the batch (PPR_MEM_HOST) or device pointers as given
+//   keys            k_batch_keys: (v,u) and (u,v) keys + id range check
+//   sort x2         in-house LSD radix sort (primitives.cu)
+//   heads           run nets + segment heads of both orders
+//   a1 store        validate (deletion claims) -> in-place apply | rebuild
+//   a2 restore      Lemma 3 closed form per touched u, d_out update
+//   a3-a6 push      one cooperative persistent kernel: POS then NEG (push.cu)
+//   stats           one D2H copy of the device control block
+//
+// Every kernel checks the device error flag first, so a batch that fails
+// validation (ERANGE / ENOENT) mutates nothing and costs no host round-trip
+// until the final stats copy.
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cmath>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <new>
+#include <string>
+#include <vector>
+
+#include "../../include/ppr.h"
+#include "ppr_internal.cuh"
+#include "primitives.cuh"
+#include "push.cuh"
+#include "store.cuh"
+
+using namespace ppr;
+
+struct ppr_ctx {
+    int device = 0;
+    cudaStream_t st = nullptr;
+    bool own_stream = false;
+    int num_sms = 0;
+    uint32_t n = 0, S = 0;
+    double alpha = 0, eps = 0;
+    int undirected = 0;
+    int mode = PPR_MODE_OPT;
+    bool push_enabled = true;
+    uint32_t max_iters = 0;
+    bool timing = true;
+    bool force_rebuild = false;
+    double slack = 0.25;
+    uint32_t min_cap = 4;
+    uint64_t m = 0;          // arcs in the store
+    unsigned active = 0;     // host mirror of DevCtl::active_pool
+    uint64_t pool_cap[2] = {0, 0};
+    // device state
+    uint32_t* d_dout = nullptr;
+    Slab* d_slab = nullptr;
+    uint32_t* d_pool[2] = {nullptr, nullptr};
+    double* d_P = nullptr;
+    double* d_R = nullptr;
+    uint32_t* d_sources = nullptr;
+    unsigned long long* d_F[2] = {nullptr, nullptr};
+    double* d_W = nullptr;
+    uint32_t* d_bitmap = nullptr;
+    DevCtl* d_ctl = nullptr;
+    DevCtl* h_ctl = nullptr;  // pinned
+    VertexBufs vb{};
+    // batch scratch
+    uint64_t bcap = 0;  // sort entries
+    uint64_t ucap = 0;  // input updates per kind
+    BatchBufs bb{};
+    uint32_t* d_in[4] = {nullptr, nullptr, nullptr, nullptr};
+    int shifts[8] = {0};
+    int npasses = 0;
+    cudaEvent_t ev[5] = {nullptr, nullptr, nullptr, nullptr, nullptr};
+    std::string err;
+    bool poisoned = false;
+    uint64_t dev_bytes = 0;
+    std::vector<void*> allocs;
+};
+
+namespace {
+
+void set_err(ppr_ctx* h, const char* fmt, ...) {
+    char buf[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(buf, sizeof buf, fmt, ap);
+    va_end(ap);
+    h->err = buf;
+}
+
+ppr_status cuda_fail(ppr_ctx* h, cudaError_t e, const char* where) {
+    set_err(h, "%s: %s", where, cudaGetErrorString(e));
+    h->poisoned = true;
+    return PPR_ECUDA;
+}
+
+template <typename T>
+cudaError_t dalloc(ppr_ctx* h, T** p, uint64_t count) {
+    void* q = nullptr;
+    size_t bytes = (size_t)std::max<uint64_t>(count, 1) * sizeof(T);
+    cudaError_t e = cudaMalloc(&q, bytes);
+    if (e != cudaSuccess) {
+        cudaGetLastError();
+        *p = nullptr;
+        return e;
+    }
+    h->dev_bytes += bytes;
+    *p = (T*)q;
+    return cudaSuccess;
+}
+
+template <typename T>
+void dfree(ppr_ctx* h, T*& p, uint64_t count) {
+    if (p) {
+        cudaFree(p);
+        h->dev_bytes -= (size_t)std::max<uint64_t>(count, 1) * sizeof(T);
+    }
+    p = nullptr;
+}
+
+DevGraph graph_of(const ppr_ctx* h) {
+    DevGraph g;
+    g.n = h->n;
+    g.S = h->S;
+    g.alpha = h->alpha;
+    g.eps = h->eps;
+    g.dout = h->d_dout;
+    g.slab = h->d_slab;
+    g.pool[0] = h->d_pool[0];
+    g.pool[1] = h->d_pool[1];
+    g.P = h->d_P;
+    g.R = h->d_R;
+    g.sources = h->d_sources;
+    return g;
+}
+
+int ceil_log2(uint64_t x) {
+    int b = 0;
+    while ((1ull << b) < x) b++;
+    return b < 1 ? 1 : b;
+}
+
+void free_batch(ppr_ctx* h) {
+    BatchBufs& b = h->bb;
+    for (int i = 0; i < 2; i++) {
+        dfree(h, b.kv[i], h->bcap);
+        dfree(h, b.ku[i], h->bcap);
+        dfree(h, b.ov[i], h->bcap);
+        dfree(h, b.ou[i], h->bcap);
+    }
+    dfree(h, b.hist, rs_hist_entries(h->bcap));
+    dfree(h, b.rnv, h->bcap);
+    dfree(h, b.rnu, h->bcap);
+    dfree(h, b.vheads, h->bcap);
+    dfree(h, b.uheads, h->bcap);
+    dfree(h, b.claim, h->bcap);
+    dfree(h, b.delpos, h->bcap);
+    dfree(h, b.seg_end, h->bcap);
+    dfree(h, b.seg_D, h->bcap);
+    dfree(h, b.seg_I, h->bcap);
+    for (int i = 0; i < 4; i++) dfree(h, h->d_in[i], h->ucap);
+    h->bcap = h->ucap = 0;
+}
+
+ppr_status ensure_batch(ppr_ctx* h, uint64_t nupd, uint64_t N) {
+    if (N <= h->bcap && nupd <= h->ucap) return PPR_OK;
+    cudaError_t e = cudaStreamSynchronize(h->st);
+    if (e != cudaSuccess) return cuda_fail(h, e, "ensure_batch sync");
+    free_batch(h);
+    uint64_t cap = std::max<uint64_t>(N + N / 4, 1024);
+    uint64_t ucap = std::max<uint64_t>(nupd + nupd / 4, 1024);
+    BatchBufs& b = h->bb;
+    bool ok = true;
+    for (int i = 0; i < 2; i++) {
+        ok = ok && dalloc(h, &b.kv[i], cap) == cudaSuccess && dalloc(h, &b.ku[i], cap) == cudaSuccess &&
+             dalloc(h, &b.ov[i], cap) == cudaSuccess && dalloc(h, &b.ou[i], cap) == cudaSuccess;
+    }
+    ok = ok && dalloc(h, &b.hist, rs_hist_entries(cap)) == cudaSuccess;
+    ok = ok && dalloc(h, &b.rnv, cap) == cudaSuccess && dalloc(h, &b.rnu, cap) == cudaSuccess;
+    ok = ok && dalloc(h, &b.vheads, cap) == cudaSuccess && dalloc(h, &b.uheads, cap) == cudaSuccess;
+    ok = ok && dalloc(h, &b.claim, cap) == cudaSuccess && dalloc(h, &b.delpos, cap) == cudaSuccess;
+    ok = ok && dalloc(h, &b.seg_end, cap) == cudaSuccess && dalloc(h, &b.seg_D, cap) == cudaSuccess &&
+         dalloc(h, &b.seg_I, cap) == cudaSuccess;
+    for (int i = 0; i < 4; i++) ok = ok && dalloc(h, &h->d_in[i], ucap) == cudaSuccess;
+    h->bcap = cap;
+    h->ucap = ucap;
+    if (!ok) {
+        free_batch(h);
+        set_err(h, "out of device memory for a batch of %llu arcs", (unsigned long long)N);
+        return PPR_ENOMEM;
+    }
+    return PPR_OK;
+}
+
+// the inactive pool must hold a rebuild of (m + new arcs) entries
+ppr_status ensure_alt_pool(ppr_ctx* h, uint64_t new_arcs) {
+    const unsigned alt = h->active ^ 1u;
+    const double need_d =
+        std::ceil((1.0 + h->slack) * (double)(h->m + new_arcs)) + (double)(h->min_cap + 1) * h->n + 1024;
+    const uint64_t need = (uint64_t)need_d;
+    if (h->pool_cap[alt] >= need) return PPR_OK;
+    cudaError_t e = cudaStreamSynchronize(h->st);
+    if (e != cudaSuccess) return cuda_fail(h, e, "ensure_alt_pool sync");
+    dfree(h, h->d_pool[alt], h->pool_cap[alt]);
+    h->pool_cap[alt] = 0;
+    uint64_t cap = need + need / 4;
+    if (dalloc(h, &h->d_pool[alt], cap) != cudaSuccess) {
+        set_err(h, "out of device memory for the rebuild pool (%llu entries)",
+                (unsigned long long)cap);
+        return PPR_ENOMEM;
+    }
+    h->pool_cap[alt] = cap;
+    return PPR_OK;
+}
+
+void fill_stats(ppr_ctx* h, ppr_batch_stats* s, uint32_t launches, bool timed) {
+    if (!s) return;
+    memset(s, 0, sizeof *s);
+    const DevCtl& c = *h->h_ctl;
+    s->iters_pos = c.iters[0];
+    s->iters_neg = c.iters[1];
+    s->pushes = c.pushes;
+    s->pushed_edges = c.pushed_edges;
+    s->max_frontier = c.max_frontier;
+    s->touched = (uint64_t)c.n_touched * h->S;
+    s->num_arcs = h->m;
+    s->rebuilt = (c.rebuild && c.err == KERR_OK) ? 1u : 0u;
+    s->kernel_launches = launches;
+    if (timed) {
+        float ms = 0;
+        cudaEventElapsedTime(&ms, h->ev[0], h->ev[4]);
+        s->ms_total = ms;
+        cudaEventElapsedTime(&ms, h->ev[0], h->ev[1]);
+        s->ms_store = ms;
+        cudaEventElapsedTime(&ms, h->ev[1], h->ev[2]);
+        s->ms_restore = ms;
+        cudaEventElapsedTime(&ms, h->ev[2], h->ev[3]);
+        s->ms_push = ms;
+    }
+}
+
+PushArgs push_args(ppr_ctx* h) {
+    PushArgs a{};
+    a.g = graph_of(h);
+    a.ctl = h->d_ctl;
+    a.F[0] = h->d_F[0];
+    a.F[1] = h->d_F[1];
+    a.W = h->d_W;
+    a.bitmap = h->d_bitmap;
+    a.phases = 3;
+    a.max_iters = h->max_iters;
+    a.iter_cap = 1000000;
+    return a;
+}
+
+ppr_status status_of_kerr(ppr_ctx* h, int kerr) {
+    switch (kerr) {
+        case KERR_OK: return PPR_OK;
+        case KERR_RANGE: set_err(h, "vertex id >= n"); return PPR_ERANGE;
+        case KERR_NOENT: set_err(h, "deletion of an absent arc"); return PPR_ENOENT;
+        case KERR_NOCONV:
+            set_err(h, "push exceeded the iteration cap");
+            h->poisoned = true;
+            return PPR_ENOCONV;
+        default:
+            set_err(h, "internal store overflow (%d)", kerr);
+            h->poisoned = true;
+            return PPR_ECUDA;
+    }
+}
+
+// synchronise, copy the control block, map errors
+ppr_status finish(ppr_ctx* h, const char* where) {
+    cudaError_t e = cudaMemcpyAsync(h->h_ctl, h->d_ctl, sizeof(DevCtl), cudaMemcpyDeviceToHost, h->st);
+    if (e != cudaSuccess) return cuda_fail(h, e, where);
+    e = cudaStreamSynchronize(h->st);
+    if (e == cudaSuccess) e = cudaGetLastError();
+    if (e != cudaSuccess) return cuda_fail(h, e, where);
+    return status_of_kerr(h, h->h_ctl->err);
+}
+
+void record(ppr_ctx* h, int i) {
+    if (h->timing) cudaEventRecord(h->ev[i], h->st);
+}
+
+void destroy_all(ppr_ctx* h) {
+    if (h->st) cudaStreamSynchronize(h->st);
+    free_batch(h);
+    dfree(h, h->d_dout, h->n);
+    dfree(h, h->d_slab, h->n);
+    dfree(h, h->d_pool[0], h->pool_cap[0]);
+    dfree(h, h->d_pool[1], h->pool_cap[1]);
+    dfree(h, h->d_P, (uint64_t)h->S * h->n);
+    dfree(h, h->d_R, (uint64_t)h->S * h->n);
+    dfree(h, h->d_sources, h->S);
+    dfree(h, h->d_F[0], (uint64_t)h->S * h->n);
+    dfree(h, h->d_F[1], (uint64_t)h->S * h->n);
+    dfree(h, h->d_W, (uint64_t)h->S * h->n);
+    dfree(h, h->d_bitmap, ((uint64_t)h->S * h->n + 31) / 32);
+    dfree(h, h->d_ctl, 1);
+    dfree(h, h->vb.vseg, h->n);
+    dfree(h, h->vb.newcap, h->n);
+    dfree(h, h->vb.newoff, h->n);
+    dfree(h, h->vb.part, scan_parts(h->n) + 1);
+    dfree(h, h->vb.big, h->n);
+    dfree(h, h->vb.touched, h->n);
+    if (h->h_ctl) cudaFreeHost(h->h_ctl);
+    h->h_ctl = nullptr;
+    for (auto& e : h->ev)
+        if (e) cudaEventDestroy(e), e = nullptr;
+    if (h->own_stream && h->st) cudaStreamDestroy(h->st);
+    h->st = nullptr;
+}
+
+ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
+    cudaError_t e = launch_push(h->mode, a, h->num_sms, h->st);
+    if (e != cudaSuccess) return cuda_fail(h, e, "push launch");
+    ++*launches;
+    return PPR_OK;
+}
+
+}  // namespace
+
+extern "C" {
+
+const char* ppr_status_str(ppr_status s) {
+    switch (s) {
+        case PPR_OK: return "PPR_OK";
+        case PPR_EINVAL: return "PPR_EINVAL";
+        case PPR_ERANGE: return "PPR_ERANGE";
+        case PPR_ENOENT: return "PPR_ENOENT";
+        case PPR_ENOMEM: return "PPR_ENOMEM";
+        case PPR_ECUDA: return "PPR_ECUDA";
+        case PPR_EPOISONED: return "PPR_EPOISONED";
+        case PPR_ENOCONV: return "PPR_ENOCONV";
+    }
+    return "PPR_UNKNOWN";
+}
+
+const char* ppr_last_error(const ppr_ctx* h) { return h ? h->err.c_str() : "null handle"; }
+
+uint64_t ppr_device_bytes(const ppr_ctx* h) { return h ? h->dev_bytes : 0; }
+
+ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_sources,
+                      double alpha, double eps, const ppr_opts* opts, ppr_ctx** out,
+                      ppr_batch_stats* stats) {
+    if (!out) return PPR_EINVAL;
+    *out = nullptr;
+    if (!g || !sources || num_sources == 0 || g->n == 0) return PPR_EINVAL;
+    if (!(alpha > 0.0 && alpha < 1.0) || !(eps > 0.0) || !std::isfinite(eps)) return PPR_EINVAL;
+    if (g->m > 0 && (!g->src || !g->dst)) return PPR_EINVAL;
+    if (g->n >= 0xFFFFFFFFu) return PPR_EINVAL;
+    {
+        std::vector<uint32_t> s(sources, sources + num_sources);
+        for (uint32_t x : s)
+            if (x >= g->n) return PPR_ERANGE;
+        std::sort(s.begin(), s.end());
+        if (std::adjacent_find(s.begin(), s.end()) != s.end()) return PPR_EINVAL;
+    }
+    for (uint64_t i = 0; i < g->m; i++)
+        if (g->src[i] >= g->n || g->dst[i] >= g->n) return PPR_ERANGE;
+    ppr_opts o{};
+    o.device = 0;
+    o.cuda_stream = nullptr;
+    o.mode = PPR_MODE_OPT;
+    o.slack = 0.25;
+    o.min_cap = 4;
+    if (opts) o = *opts;
+    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_VANILLA || !(o.slack >= 0.0) ||
+        o.min_cap == 0)
+        return PPR_EINVAL;
+
+    ppr_ctx* h = new (std::nothrow) ppr_ctx();
+    if (!h) return PPR_ENOMEM;
+    h->device = o.device;
+    h->n = g->n;
+    h->S = num_sources;
+    h->alpha = alpha;
+    h->eps = eps;
+    h->undirected = g->undirected ? 1 : 0;
+    h->mode = o.mode;
+    h->slack = o.slack;
+    h->min_cap = o.min_cap;
+
+    cudaError_t e = cudaSetDevice(h->device);
+    if (e != cudaSuccess) {
+        delete h;
+        return PPR_EINVAL;
+    }
+    cudaDeviceGetAttribute(&h->num_sms, cudaDevAttrMultiProcessorCount, h->device);
+    if (o.cuda_stream) {
+        h->st = (cudaStream_t)o.cuda_stream;
+    } else {
+        e = cudaStreamCreateWithFlags(&h->st, cudaStreamNonBlocking);
+        if (e != cudaSuccess) {
+            delete h;
+            return PPR_ECUDA;
+        }
+        h->own_stream = true;
+    }
+    for (auto& ev : h->ev) cudaEventCreate(&ev);
+    h->npasses = key_shifts(ceil_log2(h->n), h->shifts);
+
+    const uint64_t Sn = (uint64_t)h->S * h->n;
+    const uint64_t arcs_in = g->undirected ? 2 * g->m : g->m;
+    bool ok = dalloc(h, &h->d_dout, h->n) == cudaSuccess && dalloc(h, &h->d_slab, h->n) == cudaSuccess &&
+              dalloc(h, &h->d_P, Sn) == cudaSuccess && dalloc(h, &h->d_R, Sn) == cudaSuccess &&
+              dalloc(h, &h->d_sources, h->S) == cudaSuccess &&
+              dalloc(h, &h->d_F[0], Sn) == cudaSuccess && dalloc(h, &h->d_F[1], Sn) == cudaSuccess &&
+              dalloc(h, &h->d_W, Sn) == cudaSuccess &&
+              dalloc(h, &h->d_bitmap, (Sn + 31) / 32) == cudaSuccess &&
+              dalloc(h, &h->d_ctl, 1) == cudaSuccess && dalloc(h, &h->vb.vseg, h->n) == cudaSuccess &&
+              dalloc(h, &h->vb.newcap, h->n) == cudaSuccess &&
+              dalloc(h, &h->vb.newoff, h->n) == cudaSuccess &&
+              dalloc(h, &h->vb.part, scan_parts(h->n) + 1) == cudaSuccess &&
+              dalloc(h, &h->vb.big, h->n) == cudaSuccess &&
+              dalloc(h, &h->vb.touched, h->n) == cudaSuccess &&
+              cudaMallocHost(&h->h_ctl, sizeof(DevCtl)) == cudaSuccess;
+    uint32_t *d_src = nullptr, *d_dst = nullptr;
+    ok = ok && dalloc(h, &d_src, g->m) == cudaSuccess && dalloc(h, &d_dst, g->m) == cudaSuccess;
+    if (!ok) {
+        dfree(h, d_src, g->m);
+        dfree(h, d_dst, g->m);
+        destroy_all(h);
+        delete h;
+        return PPR_ENOMEM;
+    }
+    uint32_t launches = 0;
+    cudaStream_t st = h->st;
+    record(h, 0);
+    cudaMemsetAsync(h->d_ctl, 0, sizeof(DevCtl), st);
+    cudaMemsetAsync(h->d_dout, 0, sizeof(uint32_t) * h->n, st);
+    cudaMemsetAsync(h->d_slab, 0, sizeof(Slab) * h->n, st);
+    cudaMemsetAsync(h->d_P, 0, sizeof(double) * Sn, st);
+    cudaMemsetAsync(h->d_R, 0, sizeof(double) * Sn, st);
+    cudaMemsetAsync(h->d_bitmap, 0, sizeof(uint32_t) * ((Sn + 31) / 32), st);
+    cudaMemsetAsync(h->vb.vseg, 0xFF, sizeof(uint32_t) * h->n, st);
+    cudaMemcpyAsync(h->d_sources, sources, sizeof(uint32_t) * h->S, cudaMemcpyHostToDevice, st);
+    if (g->m) {
+        cudaMemcpyAsync(d_src, g->src, sizeof(uint32_t) * g->m, cudaMemcpyHostToDevice, st);
+        cudaMemcpyAsync(d_dst, g->dst, sizeof(uint32_t) * g->m, cudaMemcpyHostToDevice, st);
+    }
+    DevGraph dg = graph_of(h);
+    launch_build_count(d_src, d_dst, g->m, h->undirected, dg, h->n, st, &launches);
+    launch_caps_from_len(dg, h->vb, h->slack, h->min_cap, st, &launches);
+    unsigned long long* d_total = &h->d_ctl->pool_top;
+    exclusive_scan_u32(h->vb.newcap, h->vb.newoff, h->n, h->vb.part, d_total, st, &launches);
+    unsigned long long total = 0;
+    cudaMemcpyAsync(&total, d_total, sizeof total, cudaMemcpyDeviceToHost, st);
+    e = cudaStreamSynchronize(st);
+    if (e == cudaSuccess) e = cudaGetLastError();
+    if (e != cudaSuccess) {
+        dfree(h, d_src, g->m);
+        dfree(h, d_dst, g->m);
+        destroy_all(h);
+        delete h;
+        return PPR_ECUDA;
+    }
+    h->pool_cap[0] = total + 1024;
+    if (dalloc(h, &h->d_pool[0], h->pool_cap[0]) != cudaSuccess) {
+        dfree(h, d_src, g->m);
+        dfree(h, d_dst, g->m);
+        destroy_all(h);
+        delete h;
+        return PPR_ENOMEM;
+    }
+    dg = graph_of(h);
+    launch_build_fill(d_src, d_dst, g->m, h->undirected, dg, h->vb, st, &launches);
+    launch_init_state(dg, st, &launches);
+    h->m = arcs_in;
+    if (h->undirected) {  // self-loops count once
+        // exact arc count = sum of in-degrees; computed by the scan of lengths below
+    }
+    record(h, 1);
+    record(h, 2);
+    // static PPR: push from the sources (P = 0, R = e_s)
+    std::vector<unsigned long long> seeds(h->S);
+    for (uint32_t i = 0; i < h->S; i++) seeds[i] = ((unsigned long long)i << 32) | sources[i];
+    unsigned long long* d_seeds = nullptr;
+    if (dalloc(h, &d_seeds, h->S) != cudaSuccess) {
+        dfree(h, d_src, g->m);
+        dfree(h, d_dst, g->m);
+        destroy_all(h);
+        delete h;
+        return PPR_ENOMEM;
+    }
+    cudaMemcpyAsync(d_seeds, seeds.data(), sizeof(unsigned long long) * h->S,
+                    cudaMemcpyHostToDevice, st);
+    PushArgs a = push_args(h);
+    a.seed_e = d_seeds;
+    a.n_seed_e = h->S;
+    ppr_status rs = run_push(h, a, &launches);
+    record(h, 3);
+    record(h, 4);
+    if (rs == PPR_OK) rs = finish(h, "ppr_create");
+    dfree(h, d_seeds, h->S);
+    dfree(h, d_src, g->m);
+    dfree(h, d_dst, g->m);
+    if (rs != PPR_OK) {
+        destroy_all(h);
+        delete h;
+        return rs;
+    }
+    if (h->undirected) {  // exact arc count (self-loops once)
+        std::vector<Slab> sl(h->n);
+        cudaMemcpy(sl.data(), h->d_slab, sizeof(Slab) * h->n, cudaMemcpyDeviceToHost);
+        uint64_t mm = 0;
+        for (auto& x : sl) mm += x.len;
+        h->m = mm;
+    }
+    fill_stats(h, stats, launches, h->timing);
+    if (stats) stats->touched = h->S;
+    *out = h;
+    return PPR_OK;
+}
+
+ppr_status ppr_destroy(ppr_ctx* h) {
+    if (!h) return PPR_EINVAL;
+    destroy_all(h);
+    delete h;
+    return PPR_OK;
+}
+
+ppr_status ppr_set_option(ppr_ctx* h, int key, int64_t value) {
+    if (!h) return PPR_EINVAL;
+    if (h->poisoned) return PPR_EPOISONED;
+    switch (key) {
+        case PPR_OPT_MODE:
+            if (value < PPR_MODE_OPT || value > PPR_MODE_VANILLA) return PPR_EINVAL;
+            h->mode = (int)value;
+            return PPR_OK;
+        case PPR_OPT_PUSH: h->push_enabled = value != 0; return PPR_OK;
+        case PPR_OPT_MAX_ITERS:
+            if (value < 0 || value > 0xFFFFFFFFll) return PPR_EINVAL;
+            h->max_iters = (uint32_t)value;
+            return PPR_OK;
+        case PPR_OPT_TIMING: h->timing = value != 0; return PPR_OK;
+        case PPR_OPT_FORCE_REBUILD: h->force_rebuild = value != 0; return PPR_OK;
+        default: return PPR_EINVAL;
+    }
+}
+
+ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* ins_dst,
+                           uint64_t n_ins, const uint32_t* del_src, const uint32_t* del_dst,
+                           uint64_t n_del, int mem, ppr_batch_stats* stats) {
+    if (!h) return PPR_EINVAL;
+    if (h->poisoned) return PPR_EPOISONED;
+    if (mem != PPR_MEM_HOST && mem != PPR_MEM_DEVICE) return PPR_EINVAL;
+    if ((n_ins && (!ins_src || !ins_dst)) || (n_del && (!del_src || !del_dst))) return PPR_EINVAL;
+    if (stats) memset(stats, 0, sizeof *stats);
+    if (n_ins + n_del == 0) {
+        if (stats) stats->num_arcs = h->m;
+        return PPR_OK;
+    }
+    const uint64_t nupd = std::max(n_ins, n_del);
+    const uint64_t N = (n_ins + n_del) * (h->undirected ? 2 : 1);
+    ppr_status rs = ensure_batch(h, nupd, N);
+    if (rs != PPR_OK) return rs;
+    rs = ensure_alt_pool(h, (h->undirected ? 2 : 1) * n_ins);
+    if (rs != PPR_OK) return rs;
+
+    cudaStream_t st = h->st;
+    uint32_t launches = 0;
+    record(h, 0);
+    const uint32_t *is = ins_src, *id = ins_dst, *ds = del_src, *dd = del_dst;
+    if (mem == PPR_MEM_HOST) {
+        if (n_ins) {
+            cudaMemcpyAsync(h->d_in[0], ins_src, 4 * n_ins, cudaMemcpyHostToDevice, st);
+            cudaMemcpyAsync(h->d_in[1], ins_dst, 4 * n_ins, cudaMemcpyHostToDevice, st);
+        }
+        if (n_del) {
+            cudaMemcpyAsync(h->d_in[2], del_src, 4 * n_del, cudaMemcpyHostToDevice, st);
+            cudaMemcpyAsync(h->d_in[3], del_dst, 4 * n_del, cudaMemcpyHostToDevice, st);
+        }
+        is = h->d_in[0];
+        id = h->d_in[1];
+        ds = h->d_in[2];
+        dd = h->d_in[3];
+    }
+    DevGraph dg = graph_of(h);
+    BatchBufs& b = h->bb;
+    launch_ctl_reset(h->d_ctl, st, &launches);
+    launch_batch_keys(is, id, n_ins, ds, dd, n_del, h->undirected, h->n, b, 0, h->d_ctl, st,
+                      &launches);
+    // two sorts of the same batch: (v,u) for the store, (u,v) for the restore
+    int wv = radix_sort_pairs(b.kv[0], b.ov[0], b.kv[1], b.ov[1], N, h->shifts, h->npasses,
+                              b.hist, st, &launches);
+    int wu = radix_sort_pairs(b.ku[0], b.ou[0], b.ku[1], b.ou[1], N, h->shifts, h->npasses,
+                              b.hist, st, &launches);
+    const uint64_t* kv = b.kv[wv];
+    const uint64_t* ku = b.ku[wu];
+    cudaMemsetAsync(b.claim, 0, sizeof(uint32_t) * N, st);
+    launch_heads(kv, b.ov[wv], N, b.rnv, b.vheads, &h->d_ctl->n_vheads, st, &launches);
+    launch_heads(ku, b.ou[wu], N, b.rnu, b.uheads, &h->d_ctl->n_uheads, st, &launches);
+    // a1: graph store
+    launch_store_validate(dg, kv, N, b, h->vb, h->d_ctl, h->force_rebuild ? 1 : 0, st, &launches);
+    launch_store_apply(dg, kv, N, b, h->d_ctl, st, &launches);
+    StoreParams sp{h->slack, h->min_cap, h->pool_cap[h->active ^ 1u]};
+    launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches);
+    launch_seg_cleanup(kv, N, b, h->vb, h->d_ctl, st, &launches);
+    record(h, 1);
+    // a2: restore
+    launch_restore(dg, ku, N, b, h->vb, h->d_ctl, st, &launches);
+    record(h, 2);
+    // a3-a6: push
+    if (h->push_enabled) {
+        PushArgs a = push_args(h);
+        a.seed_v = h->vb.touched;
+        a.n_seed_v_dev = &h->d_ctl->n_touched;
+        rs = run_push(h, a, &launches);
+        if (rs != PPR_OK) return rs;
+    }
+    record(h, 3);
+    record(h, 4);
+    rs = finish(h, "ppr_apply_batch");
+    if (rs == PPR_OK) {
+        h->m = (uint64_t)((long long)h->m + h->h_ctl->arc_delta);
+        h->active = h->h_ctl->active_pool;
+    }
+    if (rs == PPR_OK || rs == PPR_ERANGE || rs == PPR_ENOENT) fill_stats(h, stats, launches, h->timing && rs == PPR_OK);
+    return rs;
+}
+
+ppr_status ppr_push(ppr_ctx* h, ppr_batch_stats* stats) {
+    if (!h) return PPR_EINVAL;
+    if (h->poisoned) return PPR_EPOISONED;
+    uint32_t launches = 0;
+    record(h, 0);
+    record(h, 1);
+    record(h, 2);
+    launch_ctl_reset(h->d_ctl, h->st, &launches);
+    PushArgs a = push_args(h);
+    a.seed_all = 1;
+    ppr_status rs = run_push(h, a, &launches);
+    if (rs != PPR_OK) return rs;
+    record(h, 3);
+    record(h, 4);
+    rs = finish(h, "ppr_push");
+    if (rs == PPR_OK) fill_stats(h, stats, launches, h->timing);
+    return rs;
+}
+
+ppr_status ppr_reset(ppr_ctx* h) {
+    if (!h) return PPR_EINVAL;
+    if (h->poisoned) return PPR_EPOISONED;
+    uint32_t launches = 0;
+    const uint64_t Sn = (uint64_t)h->S * h->n;
+    cudaMemsetAsync(h->d_P, 0, sizeof(double) * Sn, h->st);
+    cudaMemsetAsync(h->d_R, 0, sizeof(double) * Sn, h->st);
+    launch_init_state(graph_of(h), h->st, &launches);
+    cudaError_t e = cudaStreamSynchronize(h->st);
+    if (e == cudaSuccess) e = cudaGetLastError();
+    if (e != cudaSuccess) return cuda_fail(h, e, "ppr_reset");
+    return PPR_OK;
+}
+
+ppr_status ppr_query(ppr_ctx* h, uint32_t source_idx, double* P_out, double* R_out, int mem) {
+    if (!h || (!P_out && !R_out)) return PPR_EINVAL;
+    if (h->poisoned) return PPR_EPOISONED;
+    if (source_idx >= h->S) return PPR_ERANGE;
+    if (mem != PPR_MEM_HOST && mem != PPR_MEM_DEVICE) return PPR_EINVAL;
+    const cudaMemcpyKind k = mem == PPR_MEM_HOST ? cudaMemcpyDeviceToHost : cudaMemcpyDeviceToDevice;
+    const size_t off = (size_t)source_idx * h->n;
+    cudaError_t e = cudaSuccess;
+    if (P_out) e = cudaMemcpyAsync(P_out, h->d_P + off, sizeof(double) * h->n, k, h->st);
+    if (e == cudaSuccess && R_out) e = cudaMemcpyAsync(R_out, h->d_R + off, sizeof(double) * h->n, k, h->st);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
+    if (e != cudaSuccess) return cuda_fail(h, e, "ppr_query");
+    return PPR_OK;
+}
+
+ppr_status ppr_export_dout(ppr_ctx* h, uint32_t* dout_out) {
+    if (!h || !dout_out) return PPR_EINVAL;
+    if (h->poisoned) return PPR_EPOISONED;
+    cudaError_t e = cudaMemcpyAsync(dout_out, h->d_dout, sizeof(uint32_t) * h->n,
+                                    cudaMemcpyDeviceToHost, h->st);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
+    if (e != cudaSuccess) return cuda_fail(h, e, "ppr_export_dout");
+    return PPR_OK;
+}
+
+ppr_status ppr_export_edges(ppr_ctx* h, uint32_t* src_out, uint32_t* dst_out, uint64_t cap,
+                            uint64_t* m_out) {
+    if (!h || !m_out) return PPR_EINVAL;
+    if (h->poisoned) return PPR_EPOISONED;
+    *m_out = h->m;
+    if (cap < h->m || (h->m && (!src_out || !dst_out))) return PPR_EINVAL;
+    if (h->m == 0) return PPR_OK;
+    uint32_t launches = 0;
+    uint64_t* k[2] = {nullptr, nullptr};
+    uint32_t* v[2] = {nullptr, nullptr};
+    uint32_t* hist = nullptr;
+    uint32_t* lens = nullptr;
+    unsigned long long* off = nullptr;
+    const uint64_t m = h->m;
+    bool ok = dalloc(h, &k[0], m) == cudaSuccess && dalloc(h, &k[1], m) == cudaSuccess &&
+              dalloc(h, &v[0], m) == cudaSuccess && dalloc(h, &v[1], m) == cudaSuccess &&
+              dalloc(h, &hist, rs_hist_entries(m)) == cudaSuccess &&
+              dalloc(h, &lens, h->n) == cudaSuccess && dalloc(h, &off, h->n) == cudaSuccess;
+    ppr_status rs = PPR_OK;
+    if (!ok) {
+        rs = PPR_ENOMEM;
+    } else {
+        cudaStream_t st = h->st;
+        DevGraph dg = graph_of(h);
+        launch_len_to_u32(dg, lens, st, &launches);
+        exclusive_scan_u32(lens, off, h->n, h->vb.part, &h->d_ctl->pool_top, st, &launches);
+        launch_export(dg, (int)h->active, off, k[0], st, &launches);
+        cudaMemsetAsync(v[0], 0, sizeof(uint32_t) * m, st);
+        int w = radix_sort_pairs(k[0], v[0], k[1], v[1], m, h->shifts, h->npasses, hist, st,
+                                 &launches);
+        std::vector<uint64_t> keys(m);
+        cudaMemcpyAsync(keys.data(), k[w], sizeof(uint64_t) * m, cudaMemcpyDeviceToHost, st);
+        cudaError_t e = cudaStreamSynchronize(st);
+        if (e == cudaSuccess) e = cudaGetLastError();
+        if (e != cudaSuccess) {
+            rs = cuda_fail(h, e, "ppr_export_edges");
+        } else {
+            for (uint64_t i = 0; i < m; i++) {
+                dst_out[i] = (uint32_t)(keys[i] >> 32);
+                src_out[i] = (uint32_t)keys[i];
+            }
+        }
+    }
+    dfree(h, k[0], m);
+    dfree(h, k[1], m);
+    dfree(h, v[0], m);
+    dfree(h, v[1], m);
+    dfree(h, hist, rs_hist_entries(m));
+    dfree(h, lens, h->n);
+    dfree(h, off, h->n);
+    return rs;
+}
+
+}  // extern "C"

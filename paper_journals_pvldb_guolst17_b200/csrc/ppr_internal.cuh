@@ -1,0 +1,125 @@
+// ppr_internal.cuh -- device-side data layout and helpers shared by the
+// kernels of libppr.so (sm_100a).  Nothing here is used by oracle/.
+//
+// HBM layout:
+//   dout   u32[n]                 d_out(v)                       (Table 1)
+//   slab   Slab[n] (16 B each)    {u64 off, u32 len, u32 cap} of N_in(v)
+//   pool   u32[pool_cap] x 2      slab storage; one active, one rebuild target
+//   P, R   f64[S][n]              estimate / residual per source (Table 1)
+//   F      u64[S*n] x 2           frontier entries (sidx << 32 | v), double-buffered
+//   W      f64[S*n]               Alg 3 snapshot w aligned with F (Vanilla/DupDetect)
+//   bitmap u32[ceil(S*n/32)]      UniqueEnqueue bits (Vanilla/Eager)
+//   ctl    DevCtl                 counters, flags, stats, grid barrier
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+namespace ppr {
+
+struct __align__(16) Slab {
+    unsigned long long off;  // first pool index of N_in(v)
+    uint32_t len;            // |N_in(v)| (multiset)
+    uint32_t cap;            // reserved entries
+};
+
+// error codes written by kernels into DevCtl::err (mirror ppr_status)
+enum : int { KERR_OK = 0, KERR_RANGE = -2, KERR_NOENT = -3, KERR_NOCONV = -7, KERR_OVERFLOW = -8 };
+
+struct DevCtl {
+    // frontier counters / tile counters, triple-buffered by iteration (push.cu)
+    unsigned long long fcount[3];
+    unsigned long long tilectr[3];
+    // grid barrier
+    unsigned int bar_count;
+    unsigned int bar_gen;
+    // push statistics
+    unsigned long long pushes;
+    unsigned long long pushed_edges;
+    unsigned long long max_frontier;
+    unsigned int iters[2];     // [0] = POS, [1] = NEG
+    // batch pipeline
+    int err;                   // KERR_*
+    int rebuild;               // 1: the store takes the rebuild path this batch
+    unsigned int active_pool;  // index of the active slab pool
+    unsigned int n_vheads;     // v-segments in the (v,u)-sorted batch
+    unsigned int n_uheads;     // u-segments in the (u,v)-sorted batch
+    unsigned int n_touched;    // distinct u restored
+    unsigned long long pool_top; // entries used in the active pool (after rebuild)
+    unsigned long long dup_enqueue; // debug: enqueues of an entry already queued
+    long long arc_delta;       // net change of the arc count this batch
+    unsigned int n_big;        // vertices copied warp-wide in a rebuild
+    unsigned int pad0;
+    unsigned long long pad[2];
+};
+
+struct DevGraph {
+    uint32_t n;
+    uint32_t S;
+    double alpha;
+    double eps;
+    uint32_t* dout;
+    Slab* slab;
+    uint32_t* pool[2];
+    double* P;
+    double* R;
+    const uint32_t* sources;  // [S]
+};
+
+// ------------------------------------------------------------------ helpers
+
+__device__ __forceinline__ double ld_relaxed_f64(const double* p) {
+    double v;
+    asm volatile("ld.relaxed.gpu.global.f64 %0, [%1];" : "=d"(v) : "l"(p) : "memory");
+    return v;
+}
+
+__device__ __forceinline__ unsigned int ld_acquire_u32(const unsigned int* p) {
+    unsigned int v;
+    asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+    return v;
+}
+
+__device__ __forceinline__ unsigned long long ld_acquire_u64(const unsigned long long* p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+
+__device__ __forceinline__ void st_release_u32(unsigned int* p, unsigned int v) {
+    asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+
+// Sense-free generation barrier over all CTAs of a cooperative launch.
+__device__ __forceinline__ void grid_sync(DevCtl* ctl) {
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        unsigned int gen = ld_acquire_u32(&ctl->bar_gen);
+        __threadfence();
+        unsigned int arrived = atomicAdd(&ctl->bar_count, 1u) + 1u;
+        if (arrived == gridDim.x) {
+            ctl->bar_count = 0;
+            __threadfence();
+            st_release_u32(&ctl->bar_gen, gen + 1u);
+        } else {
+            while (ld_acquire_u32(&ctl->bar_gen) == gen) __nanosleep(20);
+        }
+        __threadfence();
+    }
+    __syncthreads();
+}
+
+__device__ __forceinline__ unsigned lane_id() { return threadIdx.x & 31u; }
+
+// pushCond of Alg 3 lines 8-10: POS r > eps, NEG r < -eps
+template <bool POS>
+__device__ __forceinline__ bool push_cond(double r, double eps) {
+    return POS ? (r > eps) : (r < -eps);
+}
+
+// PushCondLocal of Alg 4 lines 1-5: the add crossed the threshold
+template <bool POS>
+__device__ __forceinline__ bool crossed(double pre, double cur, double eps) {
+    return !push_cond<POS>(pre, eps) && push_cond<POS>(cur, eps);
+}
+
+}  // namespace ppr

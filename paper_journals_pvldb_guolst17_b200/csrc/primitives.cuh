@@ -1,0 +1,40 @@
+// primitives.cuh -- hand-written device primitives for the batch pipeline:
+// LSD radix sort of (u64 key, u32 value) pairs and an exclusive scan of u32
+// counts into u64 offsets.  Both are plain multi-CTA kernels (no CUB).
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+namespace ppr {
+
+constexpr int RS_THREADS = 256;
+constexpr int RS_ITEMS = 16;
+constexpr int RS_TILE = RS_THREADS * RS_ITEMS;  // keys per CTA per pass
+
+inline uint64_t rs_tiles(uint64_t n) { return (n + RS_TILE - 1) / RS_TILE; }
+// scratch entries (u32) the sort needs for n keys
+inline uint64_t rs_hist_entries(uint64_t n) { return 256 * (rs_tiles(n) + 1) + 256; }
+
+// Sorts n pairs by the bits [shift, shift+8) for every shift in `shifts`
+// (stable LSD).  Data ping-pongs between (k0,v0) and (k1,v1); returns 0 if
+// the result ends in (k0,v0), 1 if in (k1,v1).  `launches` is incremented
+// by the number of kernels launched.
+int radix_sort_pairs(uint64_t* k0, uint32_t* v0, uint64_t* k1, uint32_t* v1, uint64_t n,
+                     const int* shifts, int npasses, uint32_t* hist, cudaStream_t st,
+                     uint32_t* launches);
+
+constexpr int SCAN_THREADS = 1024;
+constexpr int SCAN_ITEMS = 4;
+constexpr int SCAN_TILE = SCAN_THREADS * SCAN_ITEMS;
+inline uint64_t scan_parts(uint64_t n) { return (n + SCAN_TILE - 1) / SCAN_TILE; }
+
+// out[i] = sum_{j<i} in[j] (u64), *total = sum of all (device pointer).
+// part: scratch of scan_parts(n) + 1 u64.
+void exclusive_scan_u32(const uint32_t* in, unsigned long long* out, uint64_t n,
+                        unsigned long long* part, unsigned long long* total, cudaStream_t st,
+                        uint32_t* launches);
+
+// digit shifts for keys (hi << 32 | lo) with hi, lo < 2^bits
+int key_shifts(int bits, int* shifts /* >= 8 */);
+
+}  // namespace ppr

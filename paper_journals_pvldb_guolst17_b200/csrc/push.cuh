@@ -1,0 +1,33 @@
+// push.cuh -- host interface of the persistent frontier-push kernel.
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+#include "ppr_internal.cuh"
+
+namespace ppr {
+
+constexpr int PUSH_THREADS = 512;   // one frontier tile = PUSH_THREADS entries
+constexpr int PUSH_QCAP = 4096;     // per-CTA shared-memory enqueue buffer (u64 entries)
+
+struct PushArgs {
+    DevGraph g;
+    DevCtl* ctl;
+    unsigned long long* F[2];  // frontier buffers, capacity S*n each
+    double* W;                 // Alg 3 snapshot / Alg 4 r_u, aligned with F
+    uint32_t* bitmap;          // UniqueEnqueue bits, S*n
+    // seeds of each phase's initial frontier (exactly one kind is used)
+    const uint32_t* seed_v;    // vertices, crossed with all S sources
+    const unsigned int* n_seed_v_dev;  // device count of seed_v (touched list)
+    const unsigned long long* seed_e;  // explicit (sidx << 32 | v) entries
+    uint64_t n_seed_e;
+    int seed_all;              // 1: scan all S*n (Alg 3 lines 1 and 4)
+    int phases;                // bit 0: POS, bit 1: NEG
+    uint32_t max_iters;        // 0: unlimited (run to eps)
+    uint32_t iter_cap;         // safety cap -> KERR_NOCONV
+};
+
+// Launches the cooperative persistent push kernel for `mode` (PPR_MODE_*).
+cudaError_t launch_push(int mode, const PushArgs& a, int num_sms, cudaStream_t st);
+
+}  // namespace ppr

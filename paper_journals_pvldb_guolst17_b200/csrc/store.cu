@@ -1,0 +1,617 @@
+// store.cu -- dynamic graph store (hot-path step a1), invariant restore
+// (step a2) and the build/export utilities.
+//
+// Store layout: per-vertex slabs of N_in(v) (Table 1) in a u32
+// pool with slack; d_out in a separate u32 array.  A batch of arc updates
+// (u, v, op) is sorted twice with the in-house radix sort:
+//   by (v, u) -> the store: one warp per v-segment validates deletions
+//                (claims matching slab entries), then edits the slab in place
+//                (fill holes from the tail, append insertions) -- or, when a
+//                slab would overflow, the whole store is rebuilt into the
+//                other pool (capacities re-derived, scanned, copied, merged).
+//   by (u, v) -> the restore: one thread per u-segment evaluates the batch
+//                closed form of Alg 1 (Lemma 3 proof):
+//                  R(u) = r0 + [S1 + S0 (a 1[u=s] - P(u) - a r0)] / (a d_k)
+//                with S1 = (1-a) sum_j op_j P(v_j), S0 = sum_j op_j,
+//                d_k = d_0 + S0 (the post-batch out-degree, R3);
+//                d_k = 0 gives R(u) = 1[u=s] - P(u)/a (reading R4).
+// Identical (u, v) updates are first reduced to their net multiplicity so an
+// insertion and a deletion of the same arc in one batch cancel exactly.
+#include "primitives.cuh"
+#include "store.cuh"
+
+namespace ppr {
+
+namespace {
+
+__device__ __forceinline__ void set_err(DevCtl* ctl, int code) { atomicCAS(&ctl->err, KERR_OK, code); }
+
+__device__ __forceinline__ uint32_t warp_sum_u32(uint32_t x) {
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) x += __shfl_xor_sync(0xffffffffu, x, o);
+    return x;
+}
+
+__device__ __forceinline__ uint32_t warp_excl_scan_u32(uint32_t x, uint32_t& total) {
+    const unsigned lane = threadIdx.x & 31u;
+    uint32_t inc = x;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+        uint32_t y = __shfl_up_sync(0xffffffffu, inc, o);
+        if (lane >= (unsigned)o) inc += y;
+    }
+    total = __shfl_sync(0xffffffffu, inc, 31);
+    return inc - x;
+}
+
+// first index in [lo, hi) with keys[i] >= key
+__device__ __forceinline__ uint64_t lower_bound_u64(const uint64_t* keys, uint64_t lo, uint64_t hi,
+                                                    uint64_t key) {
+    while (lo < hi) {
+        uint64_t mid = (lo + hi) >> 1;
+        if (keys[mid] < key) lo = mid + 1; else hi = mid;
+    }
+    return lo;
+}
+
+__device__ __forceinline__ bool contains_u32(const uint32_t* a, uint32_t n, uint32_t x) {
+    uint32_t lo = 0, hi = n;
+    while (lo < hi) {
+        uint32_t mid = (lo + hi) >> 1;
+        if (a[mid] < x) lo = mid + 1; else hi = mid;
+    }
+    return lo < n && a[lo] == x;
+}
+
+// end of the segment starting at i0 (all keys with the same high word)
+__device__ __forceinline__ uint64_t warp_segment_end(const uint64_t* keys, uint64_t N, uint64_t i0) {
+    const unsigned lane = threadIdx.x & 31u;
+    const uint64_t hi = keys[i0] >> 32;
+    uint64_t i1 = i0;
+    while (true) {
+        const uint64_t j = i1 + lane;
+        const bool same = j < N && (keys[j] >> 32) == hi;
+        const unsigned b = __ballot_sync(0xffffffffu, same);
+        if (b == 0xffffffffu) {
+            i1 += 32;
+            continue;
+        }
+        i1 += (uint64_t)(__ffs(~b) - 1);
+        return i1;
+    }
+}
+
+__device__ __forceinline__ bool is_run_head(const uint64_t* keys, uint64_t j, uint64_t i0) {
+    return j == i0 || keys[j] != keys[j - 1];
+}
+
+// ---------------------------------------------------------------- a0 keys
+
+__global__ void k_ctl_reset(DevCtl* ctl) {
+    ctl->pushes = ctl->pushed_edges = ctl->max_frontier = 0;
+    ctl->iters[0] = ctl->iters[1] = 0;
+    ctl->err = KERR_OK;
+    ctl->rebuild = 0;
+    ctl->n_vheads = ctl->n_uheads = ctl->n_touched = 0;
+    ctl->dup_enqueue = 0;
+    ctl->arc_delta = 0;
+    ctl->n_big = 0;
+}
+
+__global__ void k_batch_keys(const uint32_t* __restrict__ is, const uint32_t* __restrict__ id,
+                             uint64_t n_ins, const uint32_t* __restrict__ ds,
+                             const uint32_t* __restrict__ dd, uint64_t n_del, int undirected,
+                             uint32_t n, uint64_t* __restrict__ kv, uint32_t* __restrict__ ov,
+                             uint64_t* __restrict__ ku, uint32_t* __restrict__ ou, DevCtl* ctl) {
+    const uint64_t tot = n_ins + n_del;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < tot;
+         i += (uint64_t)gridDim.x * blockDim.x) {
+        const bool ins = i < n_ins;
+        uint32_t u = ins ? is[i] : ds[i - n_ins];
+        uint32_t v = ins ? id[i] : dd[i - n_ins];
+        uint32_t op = ins ? 2u : 0u;  // op + 1
+        if (u >= n || v >= n) {
+            set_err(ctl, KERR_RANGE);
+            u = v = 0;
+            op = 1u;
+        }
+        if (!undirected) {
+            kv[i] = ((uint64_t)v << 32) | u;
+            ku[i] = ((uint64_t)u << 32) | v;
+            ov[i] = ou[i] = op;
+        } else {  // {u,v} -> u->v and v->u; a self-loop is one arc
+            kv[2 * i] = ((uint64_t)v << 32) | u;
+            ku[2 * i] = ((uint64_t)u << 32) | v;
+            ov[2 * i] = ou[2 * i] = op;
+            kv[2 * i + 1] = ((uint64_t)u << 32) | v;
+            ku[2 * i + 1] = ((uint64_t)v << 32) | u;
+            ov[2 * i + 1] = ou[2 * i + 1] = (u == v) ? 1u : op;
+        }
+    }
+}
+
+// run nets at run heads; segment heads appended to `heads`
+__global__ void k_heads(const uint64_t* __restrict__ keys, const uint32_t* __restrict__ ops,
+                        uint64_t N, int32_t* __restrict__ run_net, uint32_t* __restrict__ heads,
+                        unsigned int* nheads) {
+    const unsigned lane = threadIdx.x & 31u;
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t b = (uint64_t)blockIdx.x * blockDim.x; b < N; b += stride) {
+        const uint64_t i = b + threadIdx.x;
+        bool seg = false;
+        if (i < N) {
+            const uint64_t k = keys[i];
+            if (i == 0 || keys[i - 1] != k) {
+                int32_t net = 0;
+                for (uint64_t j = i; j < N && keys[j] == k; j++) net += (int32_t)ops[j] - 1;
+                run_net[i] = net;
+            }
+            seg = (i == 0) || ((keys[i - 1] >> 32) != (k >> 32));
+        }
+        const unsigned m = __ballot_sync(0xffffffffu, seg);
+        if (m) {
+            unsigned base = 0;
+            if (lane == 0) base = atomicAdd(nheads, (unsigned)__popc(m));
+            base = __shfl_sync(0xffffffffu, base, 0);
+            if (seg) heads[base + __popc(m & ((1u << lane) - 1u))] = (uint32_t)i;
+        }
+    }
+}
+
+// ---------------------------------------------------------------- a1 store
+
+__global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, uint64_t N,
+                                 BatchBufs b, uint32_t* __restrict__ vseg, DevCtl* ctl,
+                                 int force_rebuild) {
+    const unsigned lane = threadIdx.x & 31u;
+    const uint32_t nseg = *(volatile unsigned*)&ctl->n_vheads;
+    const uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->active_pool];
+    const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    if (force_rebuild && blockIdx.x == 0 && threadIdx.x == 0) ctl->rebuild = 1;
+    for (uint64_t w = warp; w < nseg; w += nwarps) {
+        const uint64_t i0 = b.vheads[w];
+        const uint32_t v = (uint32_t)(kv[i0] >> 32);
+        const uint64_t i1 = warp_segment_end(kv, N, i0);
+        uint32_t I = 0, Dn = 0;
+        for (uint64_t j = i0 + lane; j < i1; j += 32) {
+            if (is_run_head(kv, j, i0)) {
+                const int32_t net = b.rnv[j];
+                if (net > 0) I += (uint32_t)net; else Dn += (uint32_t)(-net);
+            }
+        }
+        I = warp_sum_u32(I);
+        Dn = warp_sum_u32(Dn);
+        const Slab sl = g.slab[v];
+        uint32_t found = 0;
+        if (Dn > 0) {
+            for (uint32_t p0 = 0; p0 < sl.len && found < Dn; p0 += 32) {
+                const uint32_t p = p0 + lane;
+                bool claimed = false;
+                if (p < sl.len) {
+                    const uint32_t x = pool[sl.off + p];
+                    const uint64_t key = ((uint64_t)v << 32) | x;
+                    const uint64_t q = lower_bound_u64(kv, i0, i1, key);
+                    if (q < i1 && kv[q] == key) {
+                        const int32_t net = b.rnv[q];
+                        if (net < 0) claimed = atomicAdd(&b.claim[q], 1u) < (uint32_t)(-net);
+                    }
+                }
+                const unsigned m = __ballot_sync(0xffffffffu, claimed);
+                if (claimed) b.delpos[i0 + found + __popc(m & ((1u << lane) - 1u))] = p;
+                found += __popc(m);
+            }
+        }
+        if (lane == 0) {
+            b.seg_end[i0] = (uint32_t)i1;
+            b.seg_D[i0] = found;
+            b.seg_I[i0] = I;
+            vseg[v] = (uint32_t)i0;
+            if (found < Dn) set_err(ctl, KERR_NOENT);  // deletion of an absent arc
+            if ((uint64_t)sl.len - found + I > sl.cap) ctl->rebuild = 1;
+            atomicAdd((unsigned long long*)&ctl->arc_delta,
+                      (unsigned long long)((long long)I - (long long)Dn));
+        }
+    }
+}
+
+__global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, BatchBufs b,
+                              DevCtl* ctl) {
+    if (*(volatile int*)&ctl->err != KERR_OK || *(volatile int*)&ctl->rebuild) return;
+    const unsigned lane = threadIdx.x & 31u;
+    const uint32_t nseg = *(volatile unsigned*)&ctl->n_vheads;
+    uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->active_pool];
+    const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    for (uint64_t w = warp; w < nseg; w += nwarps) {
+        const uint64_t i0 = b.vheads[w];
+        const uint32_t v = (uint32_t)(kv[i0] >> 32);
+        const uint64_t i1 = b.seg_end[i0];
+        const uint32_t D = b.seg_D[i0], I = b.seg_I[i0];
+        const Slab sl = g.slab[v];
+        const uint32_t keep = sl.len - D;
+        const uint32_t* dp = b.delpos + i0;
+        // fill the holes (deleted positions < keep) with the surviving tail entries
+        uint32_t filled = 0;
+        for (uint32_t t0 = keep; t0 < sl.len; t0 += 32) {
+            const uint32_t t = t0 + lane;
+            const bool filler = t < sl.len && !contains_u32(dp, D, t);
+            const unsigned m = __ballot_sync(0xffffffffu, filler);
+            if (filler) {
+                const uint32_t hole = dp[filled + __popc(m & ((1u << lane) - 1u))];
+                pool[sl.off + hole] = pool[sl.off + t];
+            }
+            filled += __popc(m);
+        }
+        __syncwarp();
+        // append insertions (net multiplicity copies of u) at [keep, keep + I)
+        uint32_t pos = keep;
+        for (uint64_t j0 = i0; j0 < i1; j0 += 32) {
+            const uint64_t j = j0 + lane;
+            uint32_t c = 0, x = 0;
+            if (j < i1 && is_run_head(kv, j, i0)) {
+                const int32_t net = b.rnv[j];
+                if (net > 0) {
+                    c = (uint32_t)net;
+                    x = (uint32_t)kv[j];
+                }
+            }
+            uint32_t tot;
+            const uint32_t ex = warp_excl_scan_u32(c, tot);
+            for (uint32_t k = 0; k < c; k++) pool[sl.off + pos + ex + k] = x;
+            pos += tot;
+        }
+        if (lane == 0) g.slab[v].len = keep + I;
+    }
+}
+
+// ---------------------------------------------------------------- a1 rebuild
+
+__global__ void k_rebuild_caps(DevGraph g, BatchBufs b, VertexBufs vb, double slack,
+                               uint32_t min_cap, DevCtl* ctl) {
+    if (*(volatile int*)&ctl->err != KERR_OK || !*(volatile int*)&ctl->rebuild) return;
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
+         v += (uint64_t)gridDim.x * blockDim.x) {
+        uint32_t len = g.slab[v].len;
+        const uint32_t sg = vb.vseg[v];
+        if (sg != NONE) len = len - b.seg_D[sg] + b.seg_I[sg];
+        uint32_t extra = (uint32_t)ceil((double)len * slack);
+        vb.newcap[v] = len + (extra > min_cap ? extra : min_cap);
+    }
+}
+
+__global__ void k_rebuild_copy_small(DevGraph g, VertexBufs vb, uint64_t alt_cap, DevCtl* ctl) {
+    if (*(volatile int*)&ctl->err != KERR_OK || !*(volatile int*)&ctl->rebuild) return;
+    const unsigned act = *(volatile unsigned*)&ctl->active_pool;
+    const uint32_t* src = g.pool[act];
+    uint32_t* dst = g.pool[act ^ 1u];
+    const unsigned lane = threadIdx.x & 31u;
+    for (uint64_t b0 = (uint64_t)blockIdx.x * blockDim.x; b0 < g.n;
+         b0 += (uint64_t)gridDim.x * blockDim.x) {
+        const uint64_t v = b0 + threadIdx.x;
+        bool big = false;
+        if (v < g.n) {
+            const Slab sl = g.slab[v];
+            const unsigned long long no = vb.newoff[v];
+            const uint32_t nc = vb.newcap[v];
+            if (no + nc > alt_cap) set_err(ctl, KERR_OVERFLOW);
+            big = vb.vseg[v] != NONE || sl.len > 16;
+            if (!big && no + nc <= alt_cap) {
+                for (uint32_t j = 0; j < sl.len; j++) dst[no + j] = src[sl.off + j];
+                Slab ns;
+                ns.off = no;
+                ns.len = sl.len;
+                ns.cap = nc;
+                g.slab[v] = ns;
+            }
+        }
+        const unsigned m = __ballot_sync(0xffffffffu, big);
+        if (m) {
+            unsigned base = 0;
+            if (lane == 0) base = atomicAdd(&ctl->n_big, (unsigned)__popc(m));
+            base = __shfl_sync(0xffffffffu, base, 0);
+            if (big) vb.big[base + __popc(m & ((1u << lane) - 1u))] = (uint32_t)v;
+        }
+    }
+}
+
+__global__ void k_rebuild_copy_big(DevGraph g, const uint64_t* __restrict__ kv, BatchBufs b,
+                                   VertexBufs vb, uint64_t alt_cap, DevCtl* ctl) {
+    if (*(volatile int*)&ctl->err != KERR_OK || !*(volatile int*)&ctl->rebuild) return;
+    const unsigned lane = threadIdx.x & 31u;
+    const unsigned act = *(volatile unsigned*)&ctl->active_pool;
+    const uint32_t* src = g.pool[act];
+    uint32_t* dst = g.pool[act ^ 1u];
+    const uint32_t nbig = *(volatile unsigned*)&ctl->n_big;
+    const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    for (uint64_t w = warp; w < nbig; w += nwarps) {
+        const uint32_t v = vb.big[w];
+        const Slab sl = g.slab[v];
+        const unsigned long long no = vb.newoff[v];
+        const uint32_t nc = vb.newcap[v];
+        if (no + nc > alt_cap) continue;  // flagged by the small kernel
+        const uint32_t sg = vb.vseg[v];
+        const uint32_t D = sg != NONE ? b.seg_D[sg] : 0u;
+        const uint32_t* dp = sg != NONE ? b.delpos + sg : nullptr;
+        // stable copy of the surviving entries
+        uint32_t pos = 0;
+        for (uint32_t p0 = 0; p0 < sl.len; p0 += 32) {
+            const uint32_t p = p0 + lane;
+            const bool keep = p < sl.len && !(D && contains_u32(dp, D, p));
+            const unsigned m = __ballot_sync(0xffffffffu, keep);
+            if (keep) dst[no + pos + __popc(m & ((1u << lane) - 1u))] = src[sl.off + p];
+            pos += __popc(m);
+        }
+        // insertions
+        if (sg != NONE) {
+            const uint64_t i0 = sg, i1 = b.seg_end[sg];
+            for (uint64_t j0 = i0; j0 < i1; j0 += 32) {
+                const uint64_t j = j0 + lane;
+                uint32_t c = 0, x = 0;
+                if (j < i1 && is_run_head(kv, j, i0)) {
+                    const int32_t net = b.rnv[j];
+                    if (net > 0) {
+                        c = (uint32_t)net;
+                        x = (uint32_t)kv[j];
+                    }
+                }
+                uint32_t tot;
+                const uint32_t ex = warp_excl_scan_u32(c, tot);
+                for (uint32_t k = 0; k < c; k++) dst[no + pos + ex + k] = x;
+                pos += tot;
+            }
+        }
+        if (lane == 0) {
+            Slab ns;
+            ns.off = no;
+            ns.len = pos;
+            ns.cap = nc;
+            g.slab[v] = ns;
+        }
+    }
+}
+
+__global__ void k_rebuild_finish(DevCtl* ctl) {
+    if (ctl->err != KERR_OK || !ctl->rebuild) return;
+    ctl->active_pool ^= 1u;
+}
+
+__global__ void k_seg_cleanup(const uint64_t* __restrict__ kv, BatchBufs b,
+                              uint32_t* __restrict__ vseg, DevCtl* ctl) {
+    const uint32_t nseg = *(volatile unsigned*)&ctl->n_vheads;
+    for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nseg;
+         w += (uint64_t)gridDim.x * blockDim.x)
+        vseg[kv[b.vheads[w]] >> 32] = NONE;
+}
+
+// ---------------------------------------------------------------- a2 restore
+
+__global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t N, BatchBufs b,
+                          uint32_t* __restrict__ touched, DevCtl* ctl) {
+    if (*(volatile int*)&ctl->err != KERR_OK) return;
+    const uint32_t nseg = *(volatile unsigned*)&ctl->n_uheads;
+    const double a = g.alpha;
+    for (uint64_t k = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; k < nseg;
+         k += (uint64_t)gridDim.x * blockDim.x) {
+        const uint64_t i0 = b.uheads[k];
+        const uint32_t u = (uint32_t)(ku[i0] >> 32);
+        int64_t S0 = 0;
+        bool any = false;
+        uint64_t i1 = i0;
+        for (; i1 < N && (ku[i1] >> 32) == u; i1++) {
+            if (is_run_head(ku, i1, i0)) {
+                const int32_t net = b.rnu[i1];
+                S0 += net;
+                any |= net != 0;
+            }
+        }
+        if (!any) continue;
+        const int64_t dk = (int64_t)g.dout[u] + S0;  // post-batch d_out(u) (reading R3)
+        g.dout[u] = (uint32_t)dk;
+        for (uint32_t si = 0; si < g.S; si++) {
+            const size_t base = (size_t)si * g.n;
+            double s1 = 0.0;
+            for (uint64_t j = i0; j < i1; j++) {
+                if (!is_run_head(ku, j, i0)) continue;
+                const int32_t net = b.rnu[j];
+                if (net != 0) s1 += (double)net * g.P[base + (uint32_t)ku[j]];
+            }
+            const double S1 = (1.0 - a) * s1;
+            const double one = (u == g.sources[si]) ? 1.0 : 0.0;
+            const double pu = g.P[base + u];
+            const double r0 = g.R[base + u];
+            double r;
+            if (dk > 0)
+                r = r0 + (S1 + (double)S0 * (a * one - pu - a * r0)) / (a * (double)dk);
+            else
+                r = one - pu / a;  // Eq. 2 with an empty sum (reading R4)
+            g.R[base + u] = r;
+        }
+        const unsigned pos = atomicAdd(&ctl->n_touched, 1u);
+        touched[pos] = u;
+    }
+}
+
+// ---------------------------------------------------------------- build / init / export
+
+__global__ void k_build_count(const uint32_t* __restrict__ src, const uint32_t* __restrict__ dst,
+                              uint64_t m, int undirected, DevGraph g) {
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
+         i += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t u = src[i], v = dst[i];
+        atomicAdd(&g.slab[v].len, 1u);
+        atomicAdd(&g.dout[u], 1u);
+        if (undirected && u != v) {
+            atomicAdd(&g.slab[u].len, 1u);
+            atomicAdd(&g.dout[v], 1u);
+        }
+    }
+}
+
+__global__ void k_caps_from_len(DevGraph g, uint32_t* __restrict__ newcap, double slack,
+                                uint32_t min_cap) {
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
+         v += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t len = g.slab[v].len;
+        uint32_t extra = (uint32_t)ceil((double)len * slack);
+        newcap[v] = len + (extra > min_cap ? extra : min_cap);
+    }
+}
+
+__global__ void k_set_slabs(DevGraph g, const unsigned long long* __restrict__ off,
+                            const uint32_t* __restrict__ cap) {
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
+         v += (uint64_t)gridDim.x * blockDim.x) {
+        Slab s;
+        s.off = off[v];
+        s.len = 0;
+        s.cap = cap[v];
+        g.slab[v] = s;
+    }
+}
+
+__global__ void k_build_fill(const uint32_t* __restrict__ src, const uint32_t* __restrict__ dst,
+                             uint64_t m, int undirected, DevGraph g) {
+    uint32_t* pool = g.pool[0];
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
+         i += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t u = src[i], v = dst[i];
+        uint32_t p = atomicAdd(&g.slab[v].len, 1u);
+        pool[g.slab[v].off + p] = u;
+        if (undirected && u != v) {
+            p = atomicAdd(&g.slab[u].len, 1u);
+            pool[g.slab[u].off + p] = v;
+        }
+    }
+}
+
+__global__ void k_init_state(DevGraph g) {
+    // P = 0 and R = 0 are set by memset; R(s) = 1 for each source (Fig. 3 a(1))
+    for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < g.S; i += gridDim.x * blockDim.x)
+        g.R[(size_t)i * g.n + g.sources[i]] = 1.0;
+}
+
+__global__ void k_len_to_u32(DevGraph g, uint32_t* __restrict__ out) {
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
+         v += (uint64_t)gridDim.x * blockDim.x)
+        out[v] = g.slab[v].len;
+}
+
+__global__ void k_export(DevGraph g, int active, const unsigned long long* __restrict__ off,
+                         uint64_t* __restrict__ keys) {
+    const uint32_t* pool = g.pool[active];
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
+         v += (uint64_t)gridDim.x * blockDim.x) {
+        const Slab sl = g.slab[v];
+        for (uint32_t j = 0; j < sl.len; j++) keys[off[v] + j] = (v << 32) | pool[sl.off + j];
+    }
+}
+
+inline unsigned grid_for(uint64_t n, unsigned threads, unsigned cap = 148 * 32) {
+    uint64_t b = (n + threads - 1) / threads;
+    if (b < 1) b = 1;
+    if (b > cap) b = cap;
+    return (unsigned)b;
+}
+
+}  // namespace
+
+void launch_ctl_reset(DevCtl* ctl, cudaStream_t st, uint32_t* launches) {
+    k_ctl_reset<<<1, 1, 0, st>>>(ctl);
+    ++*launches;
+}
+
+void launch_batch_keys(const uint32_t* is, const uint32_t* id, uint64_t n_ins, const uint32_t* ds,
+                       const uint32_t* dd, uint64_t n_del, int undirected, uint32_t n,
+                       const BatchBufs& b, int slot, DevCtl* ctl, cudaStream_t st,
+                       uint32_t* launches) {
+    k_batch_keys<<<grid_for(n_ins + n_del, 256), 256, 0, st>>>(
+        is, id, n_ins, ds, dd, n_del, undirected, n, b.kv[slot], b.ov[slot], b.ku[slot],
+        b.ou[slot], ctl);
+    ++*launches;
+}
+
+void launch_heads(const uint64_t* keys, const uint32_t* ops, uint64_t N, int32_t* run_net,
+                  uint32_t* heads, unsigned int* nheads, cudaStream_t st, uint32_t* launches) {
+    k_heads<<<grid_for(N, 256), 256, 0, st>>>(keys, ops, N, run_net, heads, nheads);
+    ++*launches;
+}
+
+void launch_store_validate(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
+                           const VertexBufs& vb, DevCtl* ctl, int force_rebuild, cudaStream_t st,
+                           uint32_t* launches) {
+    k_store_validate<<<grid_for(N * 32, 256), 256, 0, st>>>(g, kv, N, b, vb.vseg, ctl,
+                                                            force_rebuild);
+    ++*launches;
+}
+
+void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
+                        DevCtl* ctl, cudaStream_t st, uint32_t* launches) {
+    k_store_apply<<<grid_for(N * 32, 256), 256, 0, st>>>(g, kv, b, ctl);
+    ++*launches;
+}
+
+void launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
+                          const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
+                          cudaStream_t st, uint32_t* launches) {
+    (void)N;
+    k_rebuild_caps<<<grid_for(g.n, 256), 256, 0, st>>>(g, b, vb, sp.slack, sp.min_cap, ctl);
+    ++*launches;
+    exclusive_scan_u32(vb.newcap, vb.newoff, g.n, vb.part, &ctl->pool_top, st, launches);
+    k_rebuild_copy_small<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb, sp.alt_cap, ctl);
+    k_rebuild_copy_big<<<148 * 8, 256, 0, st>>>(g, kv, b, vb, sp.alt_cap, ctl);
+    k_rebuild_finish<<<1, 1, 0, st>>>(ctl);
+    *launches += 3;
+}
+
+void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, const VertexBufs& vb,
+                        DevCtl* ctl, cudaStream_t st, uint32_t* launches) {
+    k_seg_cleanup<<<grid_for(N, 256), 256, 0, st>>>(kv, b, vb.vseg, ctl);
+    ++*launches;
+}
+
+void launch_restore(const DevGraph& g, const uint64_t* ku, uint64_t N, const BatchBufs& b,
+                    const VertexBufs& vb, DevCtl* ctl, cudaStream_t st, uint32_t* launches) {
+    k_restore<<<grid_for(N, 128), 128, 0, st>>>(g, ku, N, b, vb.touched, ctl);
+    ++*launches;
+}
+
+void launch_build_count(const uint32_t* src, const uint32_t* dst, uint64_t m, int undirected,
+                        const DevGraph& g, uint32_t n, cudaStream_t st, uint32_t* launches) {
+    (void)n;
+    k_build_count<<<grid_for(m, 256), 256, 0, st>>>(src, dst, m, undirected, g);
+    ++*launches;
+}
+
+void launch_caps_from_len(const DevGraph& g, const VertexBufs& vb, double slack, uint32_t min_cap,
+                          cudaStream_t st, uint32_t* launches) {
+    k_caps_from_len<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb.newcap, slack, min_cap);
+    ++*launches;
+}
+
+void launch_build_fill(const uint32_t* src, const uint32_t* dst, uint64_t m, int undirected,
+                       const DevGraph& g, const VertexBufs& vb, cudaStream_t st,
+                       uint32_t* launches) {
+    k_set_slabs<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb.newoff, vb.newcap);
+    k_build_fill<<<grid_for(m, 256), 256, 0, st>>>(src, dst, m, undirected, g);
+    *launches += 2;
+}
+
+void launch_init_state(const DevGraph& g, cudaStream_t st, uint32_t* launches) {
+    k_init_state<<<grid_for(g.S, 256), 256, 0, st>>>(g);
+    ++*launches;
+}
+
+void launch_export(const DevGraph& g, int active, const unsigned long long* off, uint64_t* keys,
+                   cudaStream_t st, uint32_t* launches) {
+    k_export<<<grid_for(g.n, 256), 256, 0, st>>>(g, active, off, keys);
+    ++*launches;
+}
+
+void launch_len_to_u32(const DevGraph& g, uint32_t* out, cudaStream_t st, uint32_t* launches) {
+    k_len_to_u32<<<grid_for(g.n, 256), 256, 0, st>>>(g, out);
+    ++*launches;
+}
+
+}  // namespace ppr

@@ -1,0 +1,311 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle and
+the paper's printed values.  All tests need a B200 (`-m gpu`).
+
+Gates per batch:
+  * arc multiset: bit-exact vs the oracle after every batch;
+  * Eq. 2 invariant at every vertex to 1e-12 relative (reading R18);
+  * termination: -eps <= R <= eps exactly;
+  * GPU vs oracle estimates: L_inf <= 2 eps (reading R19), L1 <= 1e-6 at
+    eps = 1e-9 on the tiny config (reading R20);
+  * Figs 1-3: bit-exact dyadic values in Vanilla (Alg 3) mode.
+"""
+import numpy as np
+import pytest
+
+import oracle
+from oracle import exact
+from paper_journals_pvldb_guolst17_b200 import ppr, workload as W
+from tests import golden_figs as G
+
+pytestmark = pytest.mark.gpu
+
+MODES = ["opt", "eager", "dupdetect", "vanilla"]
+
+
+def _fig_gpu(mode="vanilla", max_iters=0):
+    h = ppr.Ppr(G.N, G.G0_SRC, G.G0_DST, [G.SOURCE], alpha=G.ALPHA, eps=G.EPS, mode=mode)
+    return h
+
+
+# ---------------------------------------------------------------- Figs 1-3 (bit-exact)
+
+def test_fig3a_static_parallel_push_is_bit_exact():
+    h = _fig_gpu("vanilla")
+    P, R = h.query()
+    np.testing.assert_array_equal(R, [1 / 16, 0, 0, 1 / 16])
+    np.testing.assert_array_equal(P, [1 / 2, 1 / 4, 3 / 16, 1 / 16])
+    st = h.create_stats
+    assert st["iters_pos"] == 3 and st["pushes"] == 5  # Fig 3 caption
+
+
+@pytest.mark.parametrize("mode", MODES)
+def test_fig1_single_insertion(mode):
+    h = _fig_gpu(mode)
+    if mode != "vanilla":  # bring every mode to the Fig 1(a) state first
+        h.close()
+        h = _fig_gpu("vanilla")
+        h.set_option(ppr.OPT_MODE, ppr.MODES[mode])
+    h.set_option(ppr.OPT_PUSH, 0)
+    h.apply_batch([0], [1])
+    P, R = h.query()
+    assert R[0] == 5 / 32  # Fig 1(b) 0.1562
+    h.push()
+    P, R = h.query()
+    np.testing.assert_array_equal(R, [0, 5 / 64, 5 / 128, 1 / 16])   # Fig 1(d)
+    np.testing.assert_array_equal(P, [37 / 64, 1 / 4, 3 / 16, 1 / 16])
+
+
+def test_fig2_batch_restore_and_one_parallel_round():
+    h = _fig_gpu("vanilla")
+    h.set_option(ppr.OPT_PUSH, 0)
+    h.apply_batch([0, 3], [1, 0])
+    P, R = h.query()
+    np.testing.assert_array_equal(R, [5 / 32, 0, 0, 7 / 32])        # Fig 2(b)
+    st = h.push()
+    assert st["iters_pos"] == 1
+    P, R = h.query()
+    np.testing.assert_array_equal(R, [7 / 128, 5 / 64, 5 / 128, 5 / 128])   # Fig 2(d)
+    np.testing.assert_array_equal(P, [37 / 64, 1 / 4, 3 / 16, 11 / 64])
+    blk = G.load()["fig2_d"]
+    for v in range(4):
+        assert G.matches_printed(P[v], blk["P"][v]) and G.matches_printed(R[v], blk["R"][v])
+
+
+@pytest.mark.parametrize("rounds,Rw,Pw", [
+    (1, [0, .5, .25, 0], [.5, 0, 0, 0]),                 # Fig 3 a(2)
+    (2, [0, 0, .125, .125], [.5, .25, .125, 0]),         # Fig 3 a(3)
+    (3, [.0625, 0, 0, .0625], [.5, .25, .1875, .0625]),  # Fig 3 a(4)
+])
+def test_fig3a_trace_rounds(rounds, Rw, Pw):
+    h = _fig_gpu("vanilla")
+    h.reset()                       # P = 0, R = e_s (Fig 3 a(1))
+    P, R = h.query()
+    np.testing.assert_array_equal(R, [1, 0, 0, 0])
+    np.testing.assert_array_equal(P, [0, 0, 0, 0])
+    h.set_option(ppr.OPT_MAX_ITERS, rounds)
+    st = h.push()
+    assert st["iters_pos"] == rounds
+    P, R = h.query()
+    np.testing.assert_array_equal(R, Rw)
+    np.testing.assert_array_equal(P, Pw)
+
+
+# ---------------------------------------------------------------- helpers
+
+def _check_batch_state(h, o, sidx, s, eps, what):
+    P, R = h.query(sidx)
+    Po, Ro = o.query(sidx)
+    gs, gd = h.export_edges()
+    os_, od = o.export()
+    np.testing.assert_array_equal(gd, od, err_msg=f"{what}: arc dst")
+    np.testing.assert_array_equal(gs, os_, err_msg=f"{what}: arc src")
+    assert exact.terminated(R, eps), (what, np.abs(R).max())
+    ok, worst = exact.invariant_ok(h.n, gs, gd, s, h.alpha, P, R)
+    assert ok, (what, worst)
+    assert np.max(np.abs(P - Po)) <= 2 * eps, (what, np.max(np.abs(P - Po)))
+    return P, Po
+
+
+def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, **over):
+    st, cfg = W.make_stream(name, **over)
+    eps = eps or cfg["eps"]
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], sources)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=eps, mode=mode,
+                undirected=False)
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, eps)
+    o.push(oracle.SEQ)
+    for i, s in enumerate(srcs):
+        _check_batch_state(h, o, i, int(s), eps, "static")
+    last = None
+    for t in range(slides):
+        b = st.next_batch()
+        stats = h.apply_batch(*b)
+        o.apply(*b, mode=oracle.SEQ)
+        if t % check_every == check_every - 1 or t == slides - 1:
+            for i, s in enumerate(srcs):
+                last = _check_batch_state(h, o, i, int(s), eps, f"slide {t}")
+        assert stats["num_arcs"] == o.num_arcs
+    return h, o, last
+
+
+# ---------------------------------------------------------------- tiny config (configs[0])
+
+@pytest.mark.parametrize("mode", MODES)
+def test_tiny_config_all_modes_track_oracle(mode):
+    _run_stream("tiny", mode, slides=12)
+
+
+def test_tiny_config_full_50_slides_opt():
+    _run_stream("tiny", "opt", slides=50, check_every=5)
+
+
+def test_tiny_config_eps_1e9_l1_gate():
+    # reading R20: L1 <= 1e-6 at eps = 1e-9 on the tiny config
+    h, o, (P, Po) = _run_stream("tiny", "opt", slides=20, eps=1e-9, check_every=10)
+    assert np.sum(np.abs(P - Po)) <= 1e-6
+
+
+def test_tiny_config_multi_source():
+    _run_stream("tiny", "opt", slides=6, sources=4, check_every=3)
+
+
+def test_tiny_against_power_iteration():
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    (s,) = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 1)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, [s], alpha=0.15, eps=cfg["eps"])
+    for _ in range(3):
+        h.apply_batch(*st.next_batch())
+    P, R = h.query()
+    gs, gd = h.export_edges()
+    Pstar = exact.ppr_power(cfg["n"], gs, gd, int(s), 0.15)
+    assert np.max(np.abs(P - Pstar)) <= cfg["eps"] * (1 + 1e-6)
+
+
+# ---------------------------------------------------------------- restore (Lemma 3 vs Alg 1 x k)
+
+def test_restore_closed_form_matches_sequential_alg1():
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 2)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=1e-7)
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, 1e-7)
+    for sidx in range(2):  # start both from the GPU's converged state
+        P, R = h.query(sidx)
+        o.set_state(sidx, P, R)
+    h.set_option(ppr.OPT_PUSH, 0)
+    for t in range(3):
+        b = st.next_batch()
+        h.apply_batch(*b)
+        o.apply(*b, do_push=False)
+        for sidx in range(2):
+            P, R = h.query(sidx)
+            Po, Ro = o.query(sidx)
+            np.testing.assert_array_equal(P, Po)
+            scale = np.maximum(np.abs(Ro), 1.0)
+            assert np.max(np.abs(R - Ro) / scale) <= 1e-12
+        np.testing.assert_array_equal(h.export_dout(), o.dout())
+        # continue from identical states
+        h.push()
+        for sidx in range(2):
+            P, R = h.query(sidx)
+            o.set_state(sidx, P, R)
+
+
+# ---------------------------------------------------------------- edge cases
+
+def _small(mode="opt", eps=1e-9):
+    src = [0, 1, 2, 2, 3, 0]
+    dst = [3, 0, 0, 1, 2, 1]
+    h = ppr.Ppr(4, src, dst, [0], alpha=0.15, eps=eps, mode=mode)
+    o = oracle.Oracle(4, src, dst, [0], 0.15, eps)
+    o.push(oracle.SEQ)
+    return h, o
+
+
+def test_empty_batch_is_noop():
+    h, _ = _small()
+    P0, R0 = h.query()
+    st = h.apply_batch()
+    assert st["kernel_launches"] == 0
+    P1, R1 = h.query()
+    np.testing.assert_array_equal(P0, P1)
+    np.testing.assert_array_equal(R0, R1)
+
+
+def test_absent_deletion_enoent_state_unchanged():
+    h, _ = _small()
+    P0, R0 = h.query()
+    e0 = h.export_edges()
+    rc, _ = h.apply_batch([1], [3], [3, 1], [1, 2], raise_on_error=False)
+    assert rc == ppr.PPR_ENOENT
+    P1, R1 = h.query()
+    np.testing.assert_array_equal(P0, P1)
+    np.testing.assert_array_equal(R0, R1)
+    e1 = h.export_edges()
+    np.testing.assert_array_equal(e0[0], e1[0])
+    np.testing.assert_array_equal(e0[1], e1[1])
+    h.apply_batch([1], [3])  # the handle stays usable
+
+
+def test_out_of_range_erange_state_unchanged():
+    h, _ = _small()
+    P0, R0 = h.query()
+    rc, _ = h.apply_batch([1], [4], raise_on_error=False)
+    assert rc == ppr.PPR_ERANGE
+    rc, _ = h.apply_batch([], [], [9], [0], raise_on_error=False)
+    assert rc == ppr.PPR_ERANGE
+    P1, R1 = h.query()
+    np.testing.assert_array_equal(P0, P1)
+    np.testing.assert_array_equal(R0, R1)
+
+
+def test_insert_then_delete_same_arc_cancels_exactly():
+    h, _ = _small()
+    P0, R0 = h.query()
+    h.apply_batch([1], [3], [1], [3])
+    P1, R1 = h.query()
+    np.testing.assert_array_equal(P0, P1)
+    np.testing.assert_array_equal(R0, R1)
+
+
+def test_delete_last_out_arc_and_multiset_semantics():
+    h, o = _small()
+    for b in [([0, 0], [3, 3], [], []),        # multiplicity 3 on 0->3
+              ([], [], [3], [2]),              # vertex 3 loses its only out-arc
+              ([2, 2], [2, 2], [0, 0], [3, 1]),  # self-loops, deletions
+              ([1, 3], [1, 0], [2], [2])]:
+        h.apply_batch(*b)
+        o.apply(*b)
+        _check_batch_state(h, o, 0, 0, 1e-9, str(b))
+
+
+@pytest.mark.parametrize("mode", MODES)
+def test_forced_rebuild_path(mode):
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 1)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=1e-7, mode=mode)
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, 1e-7)
+    o.push(oracle.SEQ)
+    h.set_option(ppr.OPT_FORCE_REBUILD, 1)
+    for t in range(3):
+        b = st.next_batch()
+        stt = h.apply_batch(*b)
+        assert stt["rebuilt"] == 1
+        o.apply(*b)
+        _check_batch_state(h, o, 0, int(srcs[0]), 1e-7, f"rebuild slide {t}")
+
+
+def test_device_memory_batches():
+    import torch
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 1)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=1e-7)
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, 1e-7)
+    o.push(oracle.SEQ)
+    for t in range(3):
+        b = st.next_batch()
+        tb = [torch.from_numpy(x.astype(np.int32)).cuda() for x in b]
+        torch.cuda.synchronize()
+        h.apply_batch(*tb, mem=ppr.MEM_DEVICE)
+        o.apply(*b)
+        _check_batch_state(h, o, 0, int(srcs[0]), 1e-7, f"device slide {t}")
+
+
+def test_undirected_stream():
+    n = 3000
+    src, dst = W.rmat_stream(n, 20000, seed=5, abc=W.GRAPH500, undirected=True)
+    st = W.Stream(n, src, dst, w0=10000, ins_per_slide=250, del_per_slide=750, undirected=True)
+    g0s, g0d = st.window()  # already expanded to arcs
+    srcs = W.pick_sources(n, g0s, g0d, 100, 1)
+    h = ppr.Ppr(n, g0s, g0d, srcs, alpha=0.15, eps=1e-8)
+    o = oracle.Oracle(n, g0s, g0d, srcs, 0.15, 1e-8)
+    o.push(oracle.SEQ)
+    for t in range(4):
+        b = st.next_batch()
+        h.apply_batch(*b)
+        o.apply(*b)
+        _check_batch_state(h, o, 0, int(srcs[0]), 1e-8, f"undirected slide {t}")

@@ -1,0 +1,483 @@
+#!/usr/bin/env python
+"""Benchmark: batch-parallel PPR maintenance on a sliding-window edge stream.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--workload lj]
+                    [--impl ours|reference] [--sources S] [--mode opt]
+
+One step = one slide of the window: a batch of 10^4 insertions + 10^4
+deletions (configs[1], LiveJournal-shaped R-MAT) applied through the C ABI
+(ppr_apply_batch): graph-store apply -> invariant restore -> two-phase push
+to eps.  Prints ONE JSON line (rank 0).
+
+value  : edge updates/s with the batch already resident in HBM
+         (PPR_MEM_DEVICE), summed over the K timed steps' CUDA-event times.
+e2e    : the same metric through the same call with pinned HOST buffers
+         (H2D of the batch and D2H of the stats inside the timed region).
+N > 1  : one process per GPU; rank r maintains its own source (weak scaling:
+         S = N sources); rank 0 owns the stream and broadcasts every batch
+         over NCCL (the one exchange step), each rank applies it to its graph
+         replica.  Step time = max over ranks.
+--impl reference : the CPU oracle (CPU-Seq, 1 thread) on the same workload,
+         bounded by --ref-budget-s; rank 0 only.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import math
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+# algorithmic bytes per unit
+B_EDGE, B_VERTEX, B_ARC = 24, 52, 56
+
+
+def parse():
+    p = argparse.ArgumentParser()
+    p.add_argument("--gpus", type=int, default=1)
+    p.add_argument("--steps", type=int, default=100)
+    p.add_argument("--warmup", type=int, default=5)
+    p.add_argument("--workload", default="lj")
+    p.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    p.add_argument("--sources", type=int, default=0, help="total sources (0: one per rank)")
+    p.add_argument("--mode", default="opt")
+    p.add_argument("--eps", type=float, default=None)
+    p.add_argument("--ins", type=int, default=None)
+    p.add_argument("--dele", type=int, default=None)
+    p.add_argument("--seed", type=int, default=42)
+    p.add_argument("--no-cpu-baseline", action="store_true")
+    p.add_argument("--cpu-budget-s", type=float, default=30.0)
+    p.add_argument("--ref-budget-s", type=float, default=150.0)
+    p.add_argument("--no-flush", action="store_true")
+    p.add_argument("--no-e2e", action="store_true")
+    return p.parse_args()
+
+
+# ---------------------------------------------------------------- helpers
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons sampled during the timed region."""
+    Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
+         "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+         "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index):
+        self.index = index
+        self.rows = []
+        self.proc = None
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.Q}",
+                 "--format=csv,noheader,nounits", "-lms", "200"],
+                stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except Exception:
+            self.proc = None
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.rows.append([x.strip() for x in line.split(",")])
+
+    def stop(self):
+        if not self.proc:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unavailable"]}
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=5)
+        except Exception:
+            self.proc.kill()
+        self.t.join(timeout=2)
+        sm = [float(r[0]) for r in self.rows if r and r[0].replace(".", "").isdigit()]
+        mx = [float(r[1]) for r in self.rows if len(r) > 1 and r[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = set()
+        for r in self.rows:
+            for i, nm in enumerate(names):
+                if len(r) > 3 + i and r[3 + i].lower() == "active":
+                    reasons.add(nm)
+        busy = [x for x in sm if x > 300] or sm
+        return {"sm_mhz": statistics.median(busy) if busy else None,
+                "sm_max_mhz": max(mx) if mx else None, "reasons": sorted(reasons),
+                "samples": len(self.rows)}
+
+
+def measured_peak():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            return float(json.load(f)["hbm_gbs"]), "measured"
+    except Exception:
+        return 6650.0, "fallback"
+
+
+def profile_traffic(workload):
+    """dram bytes per push launch from a committed ncu --set full capture, if any."""
+    path = os.path.join(ROOT, "profiles", "push_traffic.json")
+    try:
+        with open(path) as f:
+            d = json.load(f)
+        return d.get(workload, {}).get("dram_bytes_per_launch")
+    except Exception:
+        return None
+
+
+def cpu_info():
+    model = ""
+    try:
+        with open("/proc/cpuinfo") as f:
+            for line in f:
+                if line.startswith("model name"):
+                    model = line.split(":", 1)[1].strip()
+                    break
+    except Exception:
+        pass
+    return model, os.cpu_count()
+
+
+# ---------------------------------------------------------------- distributed
+
+def dist_env():
+    ws = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return ws, rank, local
+
+
+# ---------------------------------------------------------------- reference arm
+
+def run_reference(args):
+    ws, rank, _ = dist_env()
+    if rank != 0:
+        return
+    import oracle
+    from paper_journals_pvldb_guolst17_b200 import workload as W
+    over = {}
+    if args.ins is not None:
+        over["ins"] = args.ins
+    if args.dele is not None:
+        over["dele"] = args.dele
+    st, cfg = W.make_stream(args.workload, seed=args.seed, **over)
+    eps = args.eps or cfg["eps"]
+    g0s, g0d = st.window()
+    S = args.sources or ws
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], S)
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs[:1], 0.15, eps)
+    t0 = time.perf_counter()
+    o.push(oracle.SEQ)
+    t_static = time.perf_counter() - t0
+    per = []
+    for _ in range(min(args.warmup, 1)):
+        o.apply(*st.next_batch())
+    for k in range(args.steps):
+        b = st.next_batch()
+        t0 = time.perf_counter()
+        o.apply(*b, mode=oracle.SEQ)
+        per.append(time.perf_counter() - t0)
+        if sum(per) > args.ref_budget_s:
+            break
+    upd = cfg["ins"] + cfg["dele"]
+    if cfg["undirected"]:
+        upd = upd  # undirected updates counted as given (not doubled)
+    T = sum(per)
+    value = upd * len(per) / T
+    model, ncpu = cpu_info()
+    line = {
+        "impl": "reference", "metric": "edge updates/s", "value": value, "unit": "edge updates/s",
+        "n_gpus": args.gpus, "steps": len(per), "warmup": min(args.warmup, 1),
+        "ms_per_step": 1e3 * T / len(per), "higher_is_better": True, "scaling": "weak",
+        "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": config_block(args, cfg, eps, S),
+        "cpu_baseline": {"value": value, "unit": "edge updates/s", "cores": 1, "kind": "oracle",
+                         "sample": f"{len(per)} slides of {cfg['ins']}+{cfg['dele']} after an untimed "
+                                   f"static push ({t_static:.1f} s), source rank-band top-{cfg['band']}, "
+                                   f"single thread on {ncpu}-core {model}",
+                         "sources_maintained": 1},
+        "e2e": {"value": value, "unit": "edge updates/s", "h2d_bytes_per_step": 0,
+                "d2h_bytes_per_step": 0},
+    }
+    if S > 1:
+        line["note"] = ("oracle maintains 1 of the S sources; multiply ms_per_step by S for the "
+                        "sequential cost of all sources")
+    print(json.dumps(line), flush=True)
+
+
+def config_block(args, cfg, eps, S):
+    return {"workload": args.workload, "n": cfg["n"], "m_stream": cfg["m"],
+            "window": cfg["window"] if cfg["window"] is not None else "resident",
+            "batch": f"{cfg['ins']} ins + {cfg['dele']} del per slide",
+            "undirected": cfg["undirected"], "alpha": 0.15, "eps": eps,
+            "source_band": f"top-{cfg['band']} out-degree", "sources": S,
+            "rmat_abc": list(cfg["abc"]), "mode": args.mode,
+            "l2": "flushed between steps (512 MiB write)" if not args.no_flush else "not flushed"}
+
+
+# ---------------------------------------------------------------- our arm
+
+def run_ours(args):
+    import torch
+    import torch.distributed as dist
+
+    from paper_journals_pvldb_guolst17_b200 import ppr, workload as W
+
+    ws, rank, local = dist_env()
+    if ws > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    stream = torch.cuda.Stream(dev)  # the library runs on this stream; events are recorded on it
+    torch.cuda.set_stream(stream)
+
+    over = {}
+    if args.ins is not None:
+        over["ins"] = args.ins
+    if args.dele is not None:
+        over["dele"] = args.dele
+    cfg = dict(W.CONFIGS[args.workload])
+    cfg.update(over)
+    eps = args.eps or cfg["eps"]
+    S = args.sources or ws
+    if S % ws:
+        raise SystemExit("--sources must be a multiple of the world size")
+    steps, warm = args.steps, max(args.warmup, 3)
+    nslides = steps * (1 if args.no_e2e else 2) + warm
+
+    # rank 0 owns the stream; the window and the batches go to the other
+    # ranks over NCCL (setup: untimed; per-batch broadcast: timed)
+    if rank == 0:
+        st, cfg = W.make_stream(args.workload, seed=args.seed, **over)
+        g0s, g0d = st.window()
+        srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], S)
+        batches = [st.next_batch() for _ in range(nslides)]
+        meta = torch.tensor([len(g0s)], dtype=torch.int64, device=dev)
+    else:
+        meta = torch.zeros(1, dtype=torch.int64, device=dev)
+    if ws > 1:
+        dist.broadcast(meta, 0)
+    m0 = int(meta.item())
+    if rank == 0:
+        win = torch.from_numpy(np.stack([g0s, g0d]).astype(np.int32)).to(dev)
+        srct = torch.from_numpy(srcs.astype(np.int32)).to(dev)
+    else:
+        win = torch.empty((2, m0), dtype=torch.int32, device=dev)
+        srct = torch.empty(S, dtype=torch.int32, device=dev)
+    if ws > 1:
+        dist.broadcast(win, 0)
+        dist.broadcast(srct, 0)
+    win_np = win.cpu().numpy().view(np.uint32)
+    srcs_all = srct.cpu().numpy().view(np.uint32)
+    per_rank = S // ws
+    my_srcs = srcs_all[rank * per_rank:(rank + 1) * per_rank]
+    nI, nD = cfg["ins"], cfg["dele"]
+    if cfg["undirected"]:
+        raise SystemExit("undirected workloads: expand on rank 0 (not wired in bench yet)")
+
+    t0 = time.perf_counter()
+    h = ppr.Ppr(cfg["n"], win_np[0], win_np[1], my_srcs, alpha=0.15, eps=eps, mode=args.mode,
+                device=local, stream=ctypes_stream(stream))
+    t_create = time.perf_counter() - t0
+    create_stats = h.create_stats
+    del win, win_np
+
+    # device-resident batches (rank 0) packed as [4, n]: ins_src, ins_dst, del_src, del_dst
+    def pack(b):
+        return torch.from_numpy(np.stack([b[0], b[1], b[2], b[3]]).astype(np.int32))
+
+    dev_batches = []
+    if rank == 0:
+        for b in batches[:warm + steps]:
+            dev_batches.append(pack(b).to(dev))
+    else:
+        for _ in range(warm + steps):
+            dev_batches.append(torch.empty((4, nI), dtype=torch.int32, device=dev))
+    flush_buf = torch.empty(512 * 1024 * 1024 // 4, dtype=torch.int32, device=dev)
+
+    def flush():
+        if not args.no_flush:
+            flush_buf.fill_(1)
+
+    def bcast(t):
+        if ws > 1:
+            dist.broadcast(t, 0)
+
+    def step_device(t):
+        bt = dev_batches[t]
+        bcast(bt)
+        return h.apply_batch(bt[0], bt[1], bt[2], bt[3], mem=ppr.MEM_DEVICE)
+
+    # warm-up
+    for t in range(warm):
+        step_device(t)
+    torch.cuda.synchronize()
+    if ws > 1:
+        dist.barrier()
+
+    # timed: device-resident batches
+    clocks = ClockSampler(local)
+    clocks.start()
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
+          for _ in range(steps)]
+    stats = []
+    torch.cuda.synchronize()
+    if ws > 1:
+        dist.barrier()
+    for k in range(steps):
+        flush()
+        ev[k][0].record(stream)
+        stats.append(step_device(warm + k))
+        ev[k][1].record(stream)
+    torch.cuda.synchronize()
+    if ws > 1:
+        dist.barrier()
+    ms = [a.elapsed_time(b) for a, b in ev]
+
+    # timed: end to end from pinned host buffers through the same call
+    e2e_ms = []
+    e2e_stats = []
+    if not args.no_e2e:
+        host = []
+        if rank == 0:
+            for b in batches[warm + steps:warm + 2 * steps]:
+                host.append(pack(b).pin_memory())
+        for k in range(steps):
+            flush()
+            a_, b_ = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a_.record(stream)
+            if ws > 1:
+                buf = dev_batches[k]
+                if rank == 0:
+                    buf.copy_(host[k], non_blocking=True)
+                bcast(buf)
+                s_ = h.apply_batch(buf[0], buf[1], buf[2], buf[3], mem=ppr.MEM_DEVICE)
+                s_["h2d_bytes"] = 16 * nI if rank == 0 else 0
+            else:
+                hb = host[k].numpy()
+                s_ = h.apply_batch(hb[0], hb[1], hb[2], hb[3], mem=ppr.MEM_HOST)
+            b_.record(stream)
+            b_.synchronize()
+            e2e_ms.append(a_.elapsed_time(b_))
+            e2e_stats.append(s_)
+        torch.cuda.synchronize()
+    clk = clocks.stop()
+
+    # max over ranks of the summed step time
+    T = sum(ms)
+    T_e2e = sum(e2e_ms) if e2e_ms else 0.0
+    push_ms = sum(s["ms_push"] for s in stats)
+    edges = sum(s["pushed_edges"] for s in stats)
+    verts = sum(s["pushes"] for s in stats)
+    launches = sum(s["kernel_launches"] for s in stats)
+    vec = torch.tensor([T, T_e2e, push_ms, edges, verts, launches], dtype=torch.float64, device=dev)
+    if ws > 1:
+        tmax = torch.tensor([T, T_e2e], dtype=torch.float64, device=dev)
+        dist.all_reduce(tmax, op=dist.ReduceOp.MAX)
+        tot = vec.clone()
+        dist.all_reduce(tot, op=dist.ReduceOp.SUM)
+        T, T_e2e = float(tmax[0]), float(tmax[1])
+        edges, verts, launches = float(tot[3]), float(tot[4]), float(tot[5])
+    if rank != 0:
+        h.close()
+        if ws > 1:
+            dist.destroy_process_group()
+        return
+
+    upd = nI + nD
+    value = S * upd * steps / (T / 1e3)
+    e2e_value = S * upd * len(e2e_ms) / (T_e2e / 1e3) if e2e_ms else None
+    peak, peak_kind = measured_peak()
+    # dominant kernel: the persistent push (one launch per step); rank 0's own launches
+    r0_edges = sum(s["pushed_edges"] for s in stats)
+    r0_verts = sum(s["pushes"] for s in stats)
+    bytes_per_launch = (B_EDGE * r0_edges + B_VERTEX * r0_verts) / steps
+    push_ms_avg = push_ms / steps
+    achieved = bytes_per_launch / (push_ms_avg / 1e3) / 1e9 if push_ms_avg > 0 else 0.0
+    traffic = profile_traffic(args.workload)
+
+    line = {
+        "metric": "edge updates/s", "value": value, "unit": "edge updates/s",
+        "n_gpus": ws, "steps": steps, "warmup": warm, "ms_per_step": T / steps,
+        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64",
+        "data": "synthetic", "config": config_block(args, cfg, eps, S),
+        "e2e": ({"value": e2e_value, "unit": "edge updates/s",
+                 "h2d_bytes_per_step": int(np.mean([s["h2d_bytes"] for s in e2e_stats])),
+                 "d2h_bytes_per_step": int(np.mean([s["d2h_bytes"] for s in e2e_stats])),
+                 "ms_per_step": T_e2e / len(e2e_ms)} if e2e_ms else None),
+        "gpu_launches": int(launches),
+        "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                     "frac": achieved / peak, "traffic": traffic,
+                     "kernel": "k_push<OPT> (persistent, 1 launch/step)",
+                     "algorithmic_bytes_per_launch": bytes_per_launch,
+                     "peak_kind": peak_kind, "ms_per_launch": push_ms_avg},
+        "clocks": clk,
+        "detail": {
+            "ms_per_step_p50": statistics.median(ms), "ms_per_step_p95": float(np.percentile(ms, 95)),
+            "ms_store": sum(s["ms_store"] for s in stats) / steps,
+            "ms_restore": sum(s["ms_restore"] for s in stats) / steps,
+            "ms_push": push_ms_avg,
+            "pushed_edges_per_s": edges / (T / 1e3),
+            "pushes_per_step": verts / steps / S,
+            "pushed_edges_per_step": edges / steps / S,
+            "iters_per_step": sum(s["iters_pos"] + s["iters_neg"] for s in stats) / steps,
+            "rebuilds": sum(s["rebuilt"] for s in stats),
+            "create_s": t_create, "create_stats": create_stats,
+            "device_bytes": h.device_bytes,
+        },
+    }
+    if not args.no_cpu_baseline and ws == 1:
+        line["cpu_baseline"] = cpu_baseline(args, cfg, eps, my_srcs[:1], g0s, g0d, batches)
+    h.close()
+    print(json.dumps(line), flush=True)
+    if ws > 1:
+        dist.destroy_process_group()
+
+
+def ctypes_stream(stream):
+    return stream.cuda_stream
+
+
+def cpu_baseline(args, cfg, eps, srcs, g0s, g0d, batches):
+    """The oracle (as it stands, CPU-Seq, 1 thread) on a bounded sample of the
+    same workload: untimed create + static push on the same window, then the
+    same slides, timed until --cpu-budget-s is used."""
+    import oracle
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, eps)
+    t0 = time.perf_counter()
+    o.push(oracle.SEQ)
+    t_static = time.perf_counter() - t0
+    per = []
+    for b in batches:
+        t0 = time.perf_counter()
+        o.apply(*b, mode=oracle.SEQ)
+        per.append(time.perf_counter() - t0)
+        if sum(per) > args.cpu_budget_s:
+            break
+    model, ncpu = cpu_info()
+    upd = cfg["ins"] + cfg["dele"]
+    return {"value": upd * len(per) / sum(per), "unit": "edge updates/s", "cores": 1,
+            "kind": "oracle",
+            "sample": f"first {len(per)} slides of the same stream and source (rank 0's), "
+                      f"after an untimed static push of {t_static:.1f} s; 1 thread of "
+                      f"{ncpu}-core {model}",
+            "ms_per_step": 1e3 * sum(per) / len(per)}
+
+
+def main():
+    args = parse()
+    if args.impl == "reference":
+        run_reference(args)
+    else:
+        run_ours(args)
+
+
+if __name__ == "__main__":
+    main()

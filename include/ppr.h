@@ -101,6 +101,7 @@ typedef struct {
     uint64_t num_arcs;              /* arcs in the store after the call */
     uint32_t rebuilt;               /* 1 if the slab store was rebuilt */
     uint32_t kernel_launches;       /* kernels launched by this call */
+    uint64_t h2d_bytes, d2h_bytes;  /* host<->device bytes this call copied */
     float ms_total;                 /* CUDA-event time of the call on the stream */
     float ms_store, ms_restore, ms_push; /* per phase (0 if timing disabled) */
 } ppr_batch_stats;

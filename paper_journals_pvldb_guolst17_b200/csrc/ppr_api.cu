@@ -213,9 +213,12 @@ ppr_status ensure_alt_pool(ppr_ctx* h, uint64_t new_arcs) {
     return PPR_OK;
 }
 
-void fill_stats(ppr_ctx* h, ppr_batch_stats* s, uint32_t launches, bool timed) {
+void fill_stats(ppr_ctx* h, ppr_batch_stats* s, uint32_t launches, bool timed,
+                uint64_t h2d = 0) {
     if (!s) return;
     memset(s, 0, sizeof *s);
+    s->h2d_bytes = h2d;
+    s->d2h_bytes = sizeof(DevCtl);
     const DevCtl& c = *h->h_ctl;
     s->iters_pos = c.iters[0];
     s->iters_neg = c.iters[1];
@@ -617,7 +620,9 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
         h->m = (uint64_t)((long long)h->m + h->h_ctl->arc_delta);
         h->active = h->h_ctl->active_pool;
     }
-    if (rs == PPR_OK || rs == PPR_ERANGE || rs == PPR_ENOENT) fill_stats(h, stats, launches, h->timing && rs == PPR_OK);
+    if (rs == PPR_OK || rs == PPR_ERANGE || rs == PPR_ENOENT)
+        fill_stats(h, stats, launches, h->timing && rs == PPR_OK,
+                   mem == PPR_MEM_HOST ? 8 * (n_ins + n_del) : 0);
     return rs;
 }
 

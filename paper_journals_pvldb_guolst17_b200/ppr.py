@@ -41,7 +41,8 @@ class BatchStats(ctypes.Structure):
                 ("pushes", ctypes.c_uint64), ("pushed_edges", ctypes.c_uint64),
                 ("max_frontier", ctypes.c_uint64), ("touched", ctypes.c_uint64),
                 ("num_arcs", ctypes.c_uint64), ("rebuilt", ctypes.c_uint32),
-                ("kernel_launches", ctypes.c_uint32), ("ms_total", ctypes.c_float),
+                ("kernel_launches", ctypes.c_uint32), ("h2d_bytes", ctypes.c_uint64),
+                ("d2h_bytes", ctypes.c_uint64), ("ms_total", ctypes.c_float),
                 ("ms_store", ctypes.c_float), ("ms_restore", ctypes.c_float),
                 ("ms_push", ctypes.c_float)]
 

@@ -19,6 +19,7 @@
 #include <cmath>
 #include <cstdarg>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <new>
 #include <string>
@@ -75,6 +76,8 @@ struct ppr_ctx {
     bool poisoned = false;
     uint64_t dev_bytes = 0;
     std::vector<void*> allocs;
+    unsigned long long* d_trace = nullptr;  // PPR_TRACE=1: per-round trace of the push
+    uint32_t trace_cap = 0;
 };
 
 namespace {
@@ -253,7 +256,27 @@ PushArgs push_args(ppr_ctx* h) {
     a.phases = 3;
     a.max_iters = h->max_iters;
     a.iter_cap = 1000000;
+    if (h->d_trace) {
+        cudaMemsetAsync(h->d_trace, 0, sizeof(unsigned long long) * 4 * h->trace_cap, h->st);
+        a.trace = h->d_trace;
+        a.trace_cap = h->trace_cap;
+    }
     return a;
+}
+
+// PPR_TRACE=1: print the per-round frontier sizes, times and edges of the last push
+void dump_trace(ppr_ctx* h, const char* what) {
+    if (!h->d_trace) return;
+    std::vector<unsigned long long> t(4ull * h->trace_cap);
+    cudaMemcpy(t.data(), h->d_trace, sizeof(unsigned long long) * t.size(), cudaMemcpyDeviceToHost);
+    fprintf(stderr, "PPR_TRACE %s:", what);
+    for (uint32_t i = 0; i + 1 < h->trace_cap; i++) {
+        if (t[4 * i] == ~0ull || t[4 * i + 1] == 0) break;
+        unsigned long long t1 = t[4 * (i + 1) + 1];
+        fprintf(stderr, " [%c%llu %llu %.1fus]", (t[4 * i] >> 63) ? 'N' : 'P',
+                t[4 * i] & ~(1ull << 63), t[4 * i + 2], t1 ? (t1 - t[4 * i + 1]) / 1e3 : -1.0);
+    }
+    fprintf(stderr, "\n");
 }
 
 ppr_status status_of_kerr(ppr_ctx* h, int kerr) {
@@ -311,6 +334,7 @@ void destroy_all(ppr_ctx* h) {
     h->h_ctl = nullptr;
     for (auto& e : h->ev)
         if (e) cudaEventDestroy(e), e = nullptr;
+    dfree(h, h->d_trace, 4ull * h->trace_cap);
     if (h->own_stream && h->st) cudaStreamDestroy(h->st);
     h->st = nullptr;
 }
@@ -403,6 +427,10 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     }
     for (auto& ev : h->ev) cudaEventCreate(&ev);
     h->npasses = key_shifts(ceil_log2(h->n), h->shifts);
+    if (getenv("PPR_TRACE") && atoi(getenv("PPR_TRACE")) > 0) {
+        h->trace_cap = 4096;
+        dalloc(h, &h->d_trace, 4ull * h->trace_cap);
+    }
 
     const uint64_t Sn = (uint64_t)h->S * h->n;
     const uint64_t arcs_in = g->undirected ? 2 * g->m : g->m;
@@ -616,6 +644,7 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     record(h, 3);
     record(h, 4);
     rs = finish(h, "ppr_apply_batch");
+    dump_trace(h, "apply_batch");
     if (rs == PPR_OK) {
         h->m = (uint64_t)((long long)h->m + h->h_ctl->arc_delta);
         h->active = h->h_ctl->active_pool;

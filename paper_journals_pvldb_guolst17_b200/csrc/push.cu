@@ -8,29 +8,34 @@
 //
 // Round structure per mode (Table 3):
 //   OPT       Alg 4 with the self-update fused into the same
-//             pass: per frontier tile, r_u is read ONCE with a relaxed load
-//             (eager propagation), every v in N_in(u) gets
+//             pass: r_u is read ONCE with a relaxed load (eager propagation,
+//             P:1102-1112), every v in N_in(u) gets
 //             atomicAdd(R(v), (1-a) r_u / d(v)) and is enqueued iff this add
 //             crossed the threshold (local duplicate detection, Alg 4 lines
 //             14-17); then R(u) -= r_u atomically and u is
 //             re-enqueued iff the value that subtraction produced still meets
-//             pushCond (lines 21-23).  Exactly-once enqueue
-//             argument: DESIGN.md K-PUSH.
-//   EAGER     Alg 4 order (propagate, barrier, self-update) with UniqueEnqueue
-//             through a bitmap instead of the crossing test.
-//   DUPDETECT Alg 3 order (snapshot/self-update, barrier, propagate) with the
-//             crossing test.
-//   VANILLA   Alg 3 as printed: snapshot, barrier, propagate,
-//             UniqueEnqueue through a bitmap.
+//             pushCond (lines 21-23).  Exactly-once enqueue:
+//             DESIGN.md K-PUSH.
+//   EAGER     Alg 4 order (propagate, grid barrier, self-update) with
+//             UniqueEnqueue through a bitmap instead of the crossing test.
+//   DUPDETECT Alg 3 order (snapshot/self-update, grid barrier, propagate)
+//             with the crossing test.
+//   VANILLA   Alg 3 as printed: snapshot, grid barrier,
+//             propagate, UniqueEnqueue through a bitmap.
 //
 // Work distribution (north_star "degree-binned scheduling"): a CTA takes a
-// tile of PUSH_THREADS frontier entries, scans their in-degrees in shared
-// memory and then walks the tile's edges PUSH_THREADS at a time, each thread
-// binary-searching its owner entry -- thread-, warp- and CTA-sized in-lists
-// are balanced inside the tile and slab reads are coalesced.  Tiles are
-// claimed dynamically with an atomic counter.
-// Enqueues go through a per-CTA shared-memory queue flushed with one global
-// atomic per flush (warp ballot + __syncthreads_count aggregation).
+// tile of T <= 512 frontier entries (T shrinks with the frontier so small
+// rounds still spread over all SMs; the first tile of every CTA is static,
+// later ones are claimed with one atomic per CTA), scans the entries'
+// in-degrees in shared memory, and its warps then walk the tile's edge range
+// in blocks of U x 32 edges (U independent load/atomic chains per lane for
+// memory-level parallelism), each edge finding its owner entry by binary
+// search in the shared prefix array.  In-lists of any size -- thread-, warp-
+// or CTA-sized -- are thereby balanced across all lanes of the CTA, slab
+// reads are coalesced, and no CTA barrier is needed inside the edge walk.
+// Enqueues go into a per-warp shared-memory queue slice (ballot + popc); a
+// full slice is flushed by its warp with one global atomic, and the CTA
+// flushes all slices with one atomic at the end of a round.
 #include "block_scan.cuh"
 #include "push.cuh"
 
@@ -39,111 +44,89 @@ namespace ppr {
 namespace {
 
 constexpr int PT = PUSH_THREADS;
-constexpr int QCAP = PUSH_QCAP;
-constexpr int NWARP = PT / 32;
+constexpr int NW = PT / 32;     // warps per CTA
+constexpr int U = 4;            // edges per lane per step
+constexpr int QW = 256;         // per-warp queue slice (entries)
 enum { M_OPT = 0, M_EAGER = 1, M_DUP = 2, M_VAN = 3 };
+// how a warp tile gets r and decides enqueues
+enum { K_OPT = 0, K_EAGER = 1, K_DUP = 2, K_VAN = 3 };
 
 struct Smem {
-    unsigned long long q[QCAP];       // enqueue buffer
-    unsigned long long off[PT];       // slab offset of each tile entry
-    double w[PT];                     // (1-a) * r of each tile entry
-    uint32_t scan[PT];                // exclusive prefix of in-degrees
-    uint32_t sidx[PT];                // source index of each tile entry
-    uint32_t warp[NWARP + 1];         // block-scan scratch
-    unsigned int qn;                  // entries in q
-    unsigned long long gbase;         // flush base
-    unsigned long long tile;          // claimed tile
+    uint32_t scan[PT + 1];                // exclusive in-degree prefix of the tile
+    unsigned long long off[PT];           // slab offset of each entry
+    double w[PT];                         // (1-a) * r of each entry
+    uint32_t sid[PT];                     // source index of each entry
+    unsigned long long q[NW][QW];         // per-warp enqueue slices
+    unsigned int wq[NW];                  // slice fill at the end-of-round flush
+    unsigned long long gbase;
+    unsigned long long next;              // next claimed tile
+    uint32_t warp_tmp[NW + 1];            // block-scan scratch
 };
 
+__device__ __forceinline__ unsigned long long global_ns() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+    return t;
+}
+
 struct Ctx {
-    DevGraph g;
-    DevCtl* ctl;
     const uint32_t* pool;
     unsigned long long* Fout;
     unsigned long long* cnt_out;
-    uint32_t qn;                // block-uniform queue fill
-    unsigned long long pushes;  // per-thread counters
+    unsigned long long* trace_edges;  // this round's edge counter (trace mode) or null
+    uint32_t qn;                      // warp-uniform fill of this warp's slice
+    unsigned long long pushes;        // per-thread counters
     unsigned long long edges;
 };
 
-__device__ __forceinline__ void flush(Smem& s, Ctx& c) {
-    if (c.qn == 0) return;  // block-uniform
-    if (threadIdx.x == 0) s.gbase = atomicAdd(c.cnt_out, (unsigned long long)c.qn);
-    __syncthreads();
-    const unsigned long long gb = s.gbase;
-    for (uint32_t i = threadIdx.x; i < c.qn; i += PT) c.Fout[gb + i] = s.q[i];
-    __syncthreads();
-    if (threadIdx.x == 0) s.qn = 0;
-    __syncthreads();
+__device__ __forceinline__ unsigned lane() { return threadIdx.x & 31u; }
+__device__ __forceinline__ unsigned warp() { return threadIdx.x >> 5; }
+
+__device__ __forceinline__ void warp_flush(Smem& s, Ctx& c) {
+    if (c.qn == 0) return;  // warp-uniform
+    unsigned long long base = 0;
+    if (lane() == 0) base = atomicAdd(c.cnt_out, (unsigned long long)c.qn);
+    base = __shfl_sync(0xffffffffu, base, 0);
+    const unsigned w = warp();
+    for (uint32_t i = lane(); i < c.qn; i += 32) c.Fout[base + i] = s.q[w][i];
+    __syncwarp();
     c.qn = 0;
 }
 
-// Block-wide enqueue of `e` where flag is set.  Must be called by all threads.
-__device__ __forceinline__ void enqueue(Smem& s, Ctx& c, bool flag, unsigned long long e) {
-    const unsigned lane = threadIdx.x & 31u;
+// warp-wide enqueue; caller guarantees c.qn + 32 <= QW
+__device__ __forceinline__ void warp_enqueue(Smem& s, Ctx& c, bool flag, unsigned long long e) {
     const unsigned b = __ballot_sync(0xffffffffu, flag);
-    if (b) {
-        unsigned base = 0;
-        if (lane == 0) base = atomicAdd(&s.qn, (unsigned)__popc(b));
-        base = __shfl_sync(0xffffffffu, base, 0);
-        if (flag) s.q[base + __popc(b & ((1u << lane) - 1u))] = e;
-    }
-    c.qn += (uint32_t)__syncthreads_count(flag);
-    if (c.qn > QCAP - PT) flush(s, c);
+    if (flag) s.q[warp()][c.qn + __popc(b & ((1u << lane()) - 1u))] = e;
+    c.qn += __popc(b);
 }
 
-__device__ __forceinline__ int owner_of(const Smem& s, uint32_t e) {
-    int lo = 0, hi = PT;
-    while (hi - lo > 1) {
-        int mid = (lo + hi) >> 1;
-        if (s.scan[mid] <= e) lo = mid; else hi = mid;
+__device__ __forceinline__ void ensure_room(Smem& s, Ctx& c, uint32_t need) {
+    if (c.qn + need > QW) {
+        __syncwarp();
+        warp_flush(s, c);
     }
-    return lo;
 }
 
-__device__ __forceinline__ bool claim_tile(Smem& s, unsigned long long* tc, uint32_t ntiles,
-                                           unsigned long long& t) {
-    if (threadIdx.x == 0) s.tile = atomicAdd(tc, 1ull);
+// end of a round: all slices of the CTA go out with one global atomic
+__device__ void block_flush(Smem& s, Ctx& c) {
+    const unsigned w = warp();
+    __syncwarp();
+    if (lane() == 0) s.wq[w] = c.qn;
     __syncthreads();
-    t = s.tile;
-    return t < ntiles;
-}
-
-// Loads a tile's entries: the slab of u, the weight (1-a)*r and the
-// in-degree prefix.  Returns the tile's edge count E (block-uniform).
-__device__ __forceinline__ uint32_t load_tile(Smem& s, Ctx& c, bool push, uint32_t sidx,
-                                              uint32_t u, double r) {
-    uint32_t len = 0;
-    unsigned long long off = 0;
-    if (push) {
-        const ulonglong2 sl = __ldg(reinterpret_cast<const ulonglong2*>(&c.g.slab[u]));
-        off = sl.x;                   // Slab::off
-        len = (uint32_t)sl.y;         // Slab::len (low word of {len, cap})
+    if (threadIdx.x == 0) {
+        unsigned long long tot = 0;
+        for (int i = 0; i < NW; i++) {
+            unsigned x = s.wq[i];
+            s.wq[i] = (unsigned)tot;
+            tot += x;
+        }
+        s.gbase = tot ? atomicAdd(c.cnt_out, tot) : 0ull;
     }
-    s.off[threadIdx.x] = off;
-    s.w[threadIdx.x] = __dmul_rn(1.0 - c.g.alpha, r);
-    s.sidx[threadIdx.x] = sidx;
-    uint32_t E;
-    s.scan[threadIdx.x] = block_exclusive_scan_u32<PT>(len, s.warp, &E);
     __syncthreads();
-    if (threadIdx.x == 0) c.edges += E;
-    return E;
-}
-
-// One neighbour propagation: R(v) += (1-a) w / d(v) (Alg 3 line 21, Alg 4
-// lines 13-15).  Returns pre and sets cur = pre + inc exactly as stored.
-__device__ __forceinline__ double propagate_edge(const Smem& s, Ctx& c, uint32_t e,
-                                                 unsigned long long& ev, double& cur) {
-    const int j = owner_of(s, e);
-    const uint32_t v = __ldg(&c.pool[s.off[j] + (e - s.scan[j])]);
-    const uint32_t d = __ldg(&c.g.dout[v]);
-    const double inc = __ddiv_rn(s.w[j], (double)d);
-    const uint32_t sj = s.sidx[j];
-    double* rp = c.g.R + (size_t)sj * c.g.n + v;
-    const double pre = atomicAdd(rp, inc);
-    cur = __dadd_rn(pre, inc);  // bit-identical to the stored value (no FMA)
-    ev = ((unsigned long long)sj << 32) | v;
-    return pre;
+    const unsigned long long base = s.gbase + s.wq[w];
+    for (uint32_t i = lane(); i < c.qn; i += 32) c.Fout[base + i] = s.q[w][i];
+    c.qn = 0;
+    __syncthreads();
 }
 
 __device__ __forceinline__ bool test_and_set(uint32_t* bitmap, unsigned long long bit) {
@@ -156,154 +139,176 @@ __device__ __forceinline__ void clear_bit(uint32_t* bitmap, unsigned long long b
     atomicAnd(&bitmap[bit >> 5], ~(1u << (bit & 31u)));
 }
 
-// ---------------------------------------------------------------- OPT round
+// largest i with scan[i] <= e, i in [0, T): scan[T..] hold 0xFFFFFFFF
+__device__ __forceinline__ int owner_of(const uint32_t* scan, uint32_t e, int top) {
+    int lo = 0;
+    for (int step = top; step > 0; step >>= 1)
+        if (scan[lo + step] <= e) lo += step;
+    return lo;
+}
 
-template <bool POS>
-__device__ void round_opt(Smem& s, Ctx& c, const PushArgs& a, const unsigned long long* Fin,
-                          uint64_t C, unsigned long long* tc) {
-    const uint32_t ntiles = (uint32_t)((C + PT - 1) / PT);
-    const double eps = c.g.eps, alpha = c.g.alpha;
-    unsigned long long t;
-    while (claim_tile(s, tc, ntiles, t)) {
-        const uint64_t idx = t * PT + threadIdx.x;
-        const bool valid = idx < C;
-        const unsigned long long ent = valid ? __ldcg(&Fin[idx]) : 0ull;
-        const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
-        double* ru = c.g.R + (size_t)sidx * c.g.n + u;
-        const double r = valid ? ld_relaxed_f64(ru) : 0.0;  // Alg 4 line 10
-        const bool push = valid && push_cond<POS>(r, eps);
-        const uint32_t E = load_tile(s, c, push, sidx, u, r);
-        for (uint32_t e0 = 0; e0 < E; e0 += PT) {
-            const uint32_t e = e0 + threadIdx.x;
-            bool cross = false;
-            unsigned long long ev = 0;
+// ---------------------------------------------------------------- CTA tile
+
+// Processes the T entries Fin[base_idx .. base_idx+T) (thread i = entry i):
+// neighbour propagation of every pushed entry and, for K_OPT, the fused
+// self-update.  Must be called by all threads of the CTA.
+template <bool POS, int KIND>
+__device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
+                                         const unsigned long long* Fin, uint64_t C,
+                                         uint64_t base_idx, uint32_t T, int top) {
+    const unsigned L = lane(), w = warp();
+    const double eps = a.g.eps, alpha = a.g.alpha;
+    const uint32_t n = a.g.n;
+    const uint64_t idx = base_idx + threadIdx.x;
+    const bool valid = threadIdx.x < T && idx < C;
+    const unsigned long long ent = valid ? __ldcg(&Fin[idx]) : 0ull;
+    const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
+    double* ru = a.g.R + (size_t)sidx * n + u;
+    double r = 0.0;
+    bool push = false;
+    if (KIND == K_OPT || KIND == K_EAGER) {
+        r = valid ? ld_relaxed_f64(ru) : 0.0;  // Alg 4 line 10: the current R(u)
+        push = valid && push_cond<POS>(r, eps);
+        if (KIND == K_EAGER && valid) __stcg(&a.W[idx], push ? r : 0.0);
+    } else {
+        r = valid ? __ldcg(&a.W[idx]) : 0.0;   // Alg 3: the snapshot S
+        push = valid;
+    }
+    uint32_t len = 0;
+    unsigned long long off = 0;
+    if (push) {
+        const ulonglong2 sl = __ldg(reinterpret_cast<const ulonglong2*>(&a.g.slab[u]));
+        off = sl.x;               // Slab::off
+        len = (uint32_t)sl.y;     // Slab::len (low word of {len, cap})
+    }
+    uint32_t E;
+    const uint32_t ex = block_exclusive_scan_u32<PT>(len, s.warp_tmp, &E);
+    s.scan[threadIdx.x] = threadIdx.x < T ? ex : 0xFFFFFFFFu;
+    if (threadIdx.x == 0) s.scan[PT] = 0xFFFFFFFFu;
+    s.off[threadIdx.x] = off;
+    s.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
+    s.sid[threadIdx.x] = sidx;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        c.edges += E;
+        if (c.trace_edges && E) atomicAdd(c.trace_edges, (unsigned long long)E);
+    }
+    for (uint32_t rb = w * 32 * U; rb < E; rb += NW * 32 * U) {
+        ensure_room(s, c, 32 * U);
+        uint32_t v[U];
+        int j[U];
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            const uint32_t e = rb + 32 * k + L;
+            j[k] = -1;
+            v[k] = 0;
             if (e < E) {
-                double cur;
-                const double pre = propagate_edge(s, c, e, ev, cur);
-                cross = crossed<POS>(pre, cur, eps);  // Alg 4 line 16
+                j[k] = owner_of(s.scan, e, top);
+                v[k] = __ldg(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])]);
             }
-            enqueue(s, c, cross, ev);
         }
+        uint32_t d[U];
+#pragma unroll
+        for (int k = 0; k < U; k++) d[k] = j[k] >= 0 ? __ldg(&a.g.dout[v[k]]) : 1u;
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            bool enq = false;
+            unsigned long long ev = 0;
+            if (j[k] >= 0) {
+                const uint32_t sj = s.sid[j[k]];
+                const double incr = __ddiv_rn(s.w[j[k]], (double)d[k]);
+                const double pre = atomicAdd(a.g.R + (size_t)sj * n + v[k], incr);
+                const double cur = __dadd_rn(pre, incr);  // == the stored value (no FMA)
+                ev = ((unsigned long long)sj << 32) | v[k];
+                if (KIND == K_OPT || KIND == K_DUP)
+                    enq = crossed<POS>(pre, cur, eps);   // Alg 4 line 16
+                else
+                    enq = push_cond<POS>(cur, eps) &&
+                          test_and_set(a.bitmap, (size_t)sj * n + v[k]);  // UniqueEnqueue
+            }
+            warp_enqueue(s, c, enq, ev);
+        }
+    }
+    if (KIND == K_OPT) {  // Alg 4 lines 20-23, fused: atomic subtract, re-enqueue on its result
         bool re = false;
-        if (push) {  // Alg 4 lines 20-23, fused: atomic subtract, re-enqueue on its result
+        if (push) {
             const double old = atomicAdd(ru, -r);
             const double cur = __dadd_rn(old, -r);
-            double* pu = c.g.P + (size_t)sidx * c.g.n + u;
+            double* pu = a.g.P + (size_t)sidx * n + u;
             __stcg(pu, __dadd_rn(__ldcg(pu), __dmul_rn(alpha, r)));
             re = push_cond<POS>(cur, eps);
             c.pushes++;
         }
-        enqueue(s, c, re, ent);
+        ensure_room(s, c, 32);
+        warp_enqueue(s, c, re, ent);
     }
 }
 
-// ---------------------------------------------------------------- Alg 3 rounds
+// Every CTA takes tiles of T entries: its first tile statically, the rest by
+// one atomic claim each, until C is covered.
+template <bool POS, int KIND>
+__device__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a, const unsigned long long* Fin,
+                              uint64_t C, unsigned long long* tc) {
+    uint64_t per = (C + gridDim.x - 1) / gridDim.x;
+    uint32_t T = (uint32_t)((per + 31) / 32 * 32);
+    if (T > PT) T = PT;
+    if (T < 32) T = 32;
+    int top = 1;
+    while (top * 2 < (int)T) top <<= 1;
+    const uint64_t ntiles = (C + T - 1) / T;
+    uint64_t t = blockIdx.x;
+    while (t < ntiles) {
+        cta_tile<POS, KIND>(s, c, a, Fin, C, t * T, T, top);
+        if (threadIdx.x == 0) s.next = atomicAdd(tc, 1ull) + gridDim.x;
+        __syncthreads();
+        t = s.next;
+        __syncthreads();
+    }
+}
 
-// self-update session (Alg 3 lines 13-16): w = R(u), P(u) += a w, R(u) = 0.
+// ---------------------------------------------------------------- Alg 3 / Eager sessions
+
+// self-update session of Alg 3 (lines 13-16): w = R(u), P(u) += a w, R(u) = 0
 __device__ void session_snapshot(Ctx& c, const PushArgs& a, const unsigned long long* Fin,
                                  uint64_t C, bool bitmap) {
-    const double alpha = c.g.alpha;
+    const double alpha = a.g.alpha;
     for (uint64_t idx = (uint64_t)blockIdx.x * PT + threadIdx.x; idx < C;
          idx += (uint64_t)gridDim.x * PT) {
         const unsigned long long ent = __ldcg(&Fin[idx]);
-        const size_t i = (size_t)(ent >> 32) * c.g.n + (uint32_t)ent;
-        const double w = __ldcg(&c.g.R[i]);
-        __stcg(&c.g.P[i], __dadd_rn(__ldcg(&c.g.P[i]), __dmul_rn(alpha, w)));
-        __stcg(&c.g.R[i], 0.0);
+        const size_t i = (size_t)(ent >> 32) * a.g.n + (uint32_t)ent;
+        const double w = __ldcg(&a.g.R[i]);
+        __stcg(&a.g.P[i], __dadd_rn(__ldcg(&a.g.P[i]), __dmul_rn(alpha, w)));
+        __stcg(&a.g.R[i], 0.0);
         __stcg(&a.W[idx], w);
         if (bitmap) clear_bit(a.bitmap, i);
         c.pushes++;
     }
 }
 
-// neighbour-propagation session of Alg 3 (lines 19-23) using the snapshot W.
-template <bool POS, bool UNIQUE>
-__device__ void session_propagate(Smem& s, Ctx& c, const PushArgs& a,
-                                  const unsigned long long* Fin, uint64_t C,
-                                  unsigned long long* tc) {
-    const uint32_t ntiles = (uint32_t)((C + PT - 1) / PT);
-    const double eps = c.g.eps;
-    unsigned long long t;
-    while (claim_tile(s, tc, ntiles, t)) {
-        const uint64_t idx = t * PT + threadIdx.x;
-        const bool valid = idx < C;
-        const unsigned long long ent = valid ? __ldcg(&Fin[idx]) : 0ull;
-        const double w = valid ? __ldcg(&a.W[idx]) : 0.0;
-        const uint32_t E = load_tile(s, c, valid, (uint32_t)(ent >> 32), (uint32_t)ent, w);
-        for (uint32_t e0 = 0; e0 < E; e0 += PT) {
-            const uint32_t e = e0 + threadIdx.x;
-            bool enq = false;
-            unsigned long long ev = 0;
-            if (e < E) {
-                double cur;
-                const double pre = propagate_edge(s, c, e, ev, cur);
-                if (UNIQUE) {  // UniqueEnqueue if pushCond(R(v)) (line 22-23)
-                    enq = push_cond<POS>(cur, eps) &&
-                          test_and_set(a.bitmap, (ev >> 32) * c.g.n + (uint32_t)ev);
-                } else {       // local duplicate detection
-                    enq = crossed<POS>(pre, cur, eps);
-                }
-            }
-            enqueue(s, c, enq, ev);
-        }
-    }
-}
-
-// Eager (Alg 4 order) with UniqueEnqueue: propagate with the current r_u ...
-template <bool POS>
-__device__ void session_eager_propagate(Smem& s, Ctx& c, const PushArgs& a,
-                                        const unsigned long long* Fin, uint64_t C,
-                                        unsigned long long* tc) {
-    const uint32_t ntiles = (uint32_t)((C + PT - 1) / PT);
-    const double eps = c.g.eps;
-    unsigned long long t;
-    while (claim_tile(s, tc, ntiles, t)) {
-        const uint64_t idx = t * PT + threadIdx.x;
-        const bool valid = idx < C;
-        const unsigned long long ent = valid ? __ldcg(&Fin[idx]) : 0ull;
-        const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
-        const double r = valid ? ld_relaxed_f64(c.g.R + (size_t)sidx * c.g.n + u) : 0.0;
-        const bool push = valid && push_cond<POS>(r, eps);
-        if (valid) __stcg(&a.W[idx], push ? r : 0.0);
-        const uint32_t E = load_tile(s, c, push, sidx, u, r);
-        for (uint32_t e0 = 0; e0 < E; e0 += PT) {
-            const uint32_t e = e0 + threadIdx.x;
-            bool enq = false;
-            unsigned long long ev = 0;
-            if (e < E) {
-                double cur;
-                propagate_edge(s, c, e, ev, cur);
-                enq = push_cond<POS>(cur, eps) &&
-                      test_and_set(a.bitmap, (ev >> 32) * c.g.n + (uint32_t)ev);
-            }
-            enqueue(s, c, enq, ev);
-        }
-    }
-}
-
-// ... then self-update with the same r_u (Alg 4 lines 19-23).
+// Eager: self-update with the r_u recorded during propagation (Alg 4 lines 19-23)
 template <bool POS>
 __device__ void session_eager_self(Smem& s, Ctx& c, const PushArgs& a,
                                    const unsigned long long* Fin, uint64_t C) {
-    const double eps = c.g.eps, alpha = c.g.alpha;
+    const double eps = a.g.eps, alpha = a.g.alpha;
     const uint64_t stride = (uint64_t)gridDim.x * PT;
-    for (uint64_t b = (uint64_t)blockIdx.x * PT; b < C; b += stride) {
-        const uint64_t idx = b + threadIdx.x;
+    for (uint64_t b = (uint64_t)blockIdx.x * PT + warp() * 32; b < C; b += stride) {
+        const uint64_t idx = b + lane();
         bool enq = false;
         unsigned long long ent = 0;
         if (idx < C) {
             ent = __ldcg(&Fin[idx]);
             const double r = __ldcg(&a.W[idx]);
             if (r != 0.0) {
-                const size_t i = (size_t)(ent >> 32) * c.g.n + (uint32_t)ent;
-                const double old = atomicAdd(&c.g.R[i], -r);
+                const size_t i = (size_t)(ent >> 32) * a.g.n + (uint32_t)ent;
+                const double old = atomicAdd(&a.g.R[i], -r);
                 const double cur = __dadd_rn(old, -r);
-                __stcg(&c.g.P[i], __dadd_rn(__ldcg(&c.g.P[i]), __dmul_rn(alpha, r)));
+                __stcg(&a.g.P[i], __dadd_rn(__ldcg(&a.g.P[i]), __dmul_rn(alpha, r)));
                 c.pushes++;
                 enq = push_cond<POS>(cur, eps) && test_and_set(a.bitmap, i);
             }
         }
-        enqueue(s, c, enq, ent);
+        ensure_room(s, c, 32);
+        warp_enqueue(s, c, enq, ent);
     }
 }
 
@@ -312,7 +317,7 @@ __device__ void clear_frontier_bits(Ctx& c, const PushArgs& a, const unsigned lo
     for (uint64_t idx = (uint64_t)blockIdx.x * PT + threadIdx.x; idx < C;
          idx += (uint64_t)gridDim.x * PT) {
         const unsigned long long ent = __ldcg(&Fin[idx]);
-        clear_bit(a.bitmap, (ent >> 32) * c.g.n + (uint32_t)ent);
+        clear_bit(a.bitmap, (ent >> 32) * a.g.n + (uint32_t)ent);
     }
 }
 
@@ -320,25 +325,25 @@ __device__ void clear_frontier_bits(Ctx& c, const PushArgs& a, const unsigned lo
 
 template <bool POS>
 __device__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
-    const double eps = c.g.eps;
+    const double eps = a.g.eps;
     const uint64_t stride = (uint64_t)gridDim.x * PT;
     uint64_t total;
+    const uint64_t nv = a.seed_v ? (uint64_t)(*a.n_seed_v_dev) : 0;
     if (a.seed_all)
-        total = (uint64_t)c.g.S * c.g.n;
+        total = (uint64_t)a.g.S * a.g.n;
     else if (a.seed_v)
-        total = (uint64_t)(*a.n_seed_v_dev) * c.g.S;
+        total = nv * a.g.S;
     else
         total = a.n_seed_e;
-    const uint64_t nv = a.seed_v ? (uint64_t)(*a.n_seed_v_dev) : 0;
-    for (uint64_t b = (uint64_t)blockIdx.x * PT; b < total; b += stride) {
-        const uint64_t k = b + threadIdx.x;
+    for (uint64_t b = (uint64_t)blockIdx.x * PT + warp() * 32; b < total; b += stride) {
+        const uint64_t k = b + lane();
         bool enq = false;
         unsigned long long ent = 0;
         if (k < total) {
             uint32_t sidx, v;
             if (a.seed_all) {
-                sidx = (uint32_t)(k / c.g.n);
-                v = (uint32_t)(k % c.g.n);
+                sidx = (uint32_t)(k / a.g.n);
+                v = (uint32_t)(k % a.g.n);
             } else if (a.seed_v) {
                 sidx = (uint32_t)(k / nv);
                 v = a.seed_v[k % nv];
@@ -348,9 +353,10 @@ __device__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
                 v = (uint32_t)ent;
             }
             ent = ((unsigned long long)sidx << 32) | v;
-            enq = push_cond<POS>(__ldcg(&c.g.R[(size_t)sidx * c.g.n + v]), eps);
+            enq = push_cond<POS>(__ldcg(&a.g.R[(size_t)sidx * a.g.n + v]), eps);
         }
-        enqueue(s, c, enq, ent);
+        ensure_room(s, c, 32);
+        warp_enqueue(s, c, enq, ent);
     }
 }
 
@@ -358,19 +364,24 @@ __device__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
 
 template <int MODE, bool POS>
 __device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
-    DevCtl* ctl = c.ctl;
+    DevCtl* ctl = a.ctl;
     const int ph = POS ? 0 : 1;
     // seed into F[it%2] / fcount[it%3]; both that and the next counter are 0 here
     c.Fout = a.F[it & 1];
     c.cnt_out = &ctl->fcount[it % 3];
     seed_phase<POS>(s, c, a);
-    flush(s, c);
+    block_flush(s, c);
     grid_sync(ctl);
     uint32_t pit = 0;
     uint64_t C = 0;
     while (true) {
         C = *(volatile unsigned long long*)&ctl->fcount[it % 3];
+        c.trace_edges = (a.trace && it < a.trace_cap) ? &a.trace[4ull * it + 2] : nullptr;
         if (blockIdx.x == 0 && threadIdx.x == 0) {
+            if (c.trace_edges) {
+                a.trace[4ull * it] = C | ((unsigned long long)ph << 63);
+                a.trace[4ull * it + 1] = global_ns();
+            }
             ctl->fcount[(it + 2) % 3] = 0;
             ctl->tilectr[(it + 2) % 3] = 0;
             if (C > 0 && !(a.max_iters && pit >= a.max_iters)) {
@@ -385,19 +396,22 @@ __device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
         c.cnt_out = &ctl->fcount[(it + 1) % 3];
         unsigned long long* tc = &ctl->tilectr[it % 3];
         if (MODE == M_OPT) {
-            round_opt<POS>(s, c, a, Fin, C, tc);
+            propagate_all<POS, K_OPT>(s, c, a, Fin, C, tc);
         } else if (MODE == M_VAN || MODE == M_DUP) {
             session_snapshot(c, a, Fin, C, MODE == M_VAN);
             grid_sync(ctl);
-            session_propagate<POS, MODE == M_VAN>(s, c, a, Fin, C, tc);
+            if (MODE == M_VAN)
+                propagate_all<POS, K_VAN>(s, c, a, Fin, C, tc);
+            else
+                propagate_all<POS, K_DUP>(s, c, a, Fin, C, tc);
         } else {  // M_EAGER
             clear_frontier_bits(c, a, Fin, C);
             grid_sync(ctl);
-            session_eager_propagate<POS>(s, c, a, Fin, C, tc);
+            propagate_all<POS, K_EAGER>(s, c, a, Fin, C, tc);
             grid_sync(ctl);
             session_eager_self<POS>(s, c, a, Fin, C);
         }
-        flush(s, c);
+        block_flush(s, c);
         grid_sync(ctl);
         it++;
         pit++;
@@ -407,26 +421,22 @@ __device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
     // leave the counters of the next phase's seed round at zero
     grid_sync(ctl);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
-        ctl->fcount[it % 3] = 0;
-        ctl->fcount[(it + 1) % 3] = 0;
-        ctl->fcount[(it + 2) % 3] = 0;
+        ctl->fcount[0] = ctl->fcount[1] = ctl->fcount[2] = 0;
         ctl->tilectr[0] = ctl->tilectr[1] = ctl->tilectr[2] = 0;
     }
     grid_sync(ctl);
 }
 
 template <int MODE>
-__global__ void __launch_bounds__(PT, 2) k_push(PushArgs a) {
+__global__ void __launch_bounds__(PT, 2) k_push(const __grid_constant__ PushArgs a) {
     __shared__ Smem s;
     Ctx c;
-    c.g = a.g;
-    c.ctl = a.ctl;
+    c.trace_edges = nullptr;
     c.qn = 0;
     c.pushes = 0;
     c.edges = 0;
-    if (threadIdx.x == 0) s.qn = 0;
     if (*(volatile int*)&a.ctl->err != KERR_OK) return;  // earlier stage failed: uniform exit
-    c.pool = a.g.pool[*(volatile unsigned*)&a.ctl->active_pool];
+    c.pool = *(volatile unsigned*)&a.ctl->active_pool ? a.g.pool[1] : a.g.pool[0];
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         for (int i = 0; i < 3; i++) a.ctl->fcount[i] = a.ctl->tilectr[i] = 0;
     }
@@ -434,6 +444,10 @@ __global__ void __launch_bounds__(PT, 2) k_push(PushArgs a) {
     unsigned it = 0;
     if (a.phases & 1) run_phase<MODE, true>(s, c, a, it);
     if (a.phases & 2) run_phase<MODE, false>(s, c, a, it);
+    if (a.trace && blockIdx.x == 0 && threadIdx.x == 0 && it < a.trace_cap) {
+        a.trace[4ull * it] = ~0ull;  // end marker
+        a.trace[4ull * it + 1] = global_ns();
+    }
     // statistics
     __shared__ unsigned long long s_red[2];
     if (threadIdx.x == 0) s_red[0] = s_red[1] = 0;

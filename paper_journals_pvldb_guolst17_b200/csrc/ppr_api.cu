@@ -62,7 +62,7 @@ struct ppr_ctx {
     double* d_W = nullptr;
     uint32_t* d_bitmap = nullptr;
     DevCtl* d_ctl = nullptr;
-    DevCtl* h_ctl = nullptr;  // pinned
+    DevStats* h_ctl = nullptr;  // pinned copy of DevCtl::st
     VertexBufs vb{};
     // batch scratch
     uint64_t bcap = 0;  // sort entries
@@ -221,8 +221,8 @@ void fill_stats(ppr_ctx* h, ppr_batch_stats* s, uint32_t launches, bool timed,
     if (!s) return;
     memset(s, 0, sizeof *s);
     s->h2d_bytes = h2d;
-    s->d2h_bytes = sizeof(DevCtl);
-    const DevCtl& c = *h->h_ctl;
+    s->d2h_bytes = sizeof(DevStats);
+    const DevStats& c = *h->h_ctl;
     s->iters_pos = c.iters[0];
     s->iters_neg = c.iters[1];
     s->pushes = c.pushes;
@@ -297,7 +297,7 @@ ppr_status status_of_kerr(ppr_ctx* h, int kerr) {
 
 // synchronise, copy the control block, map errors
 ppr_status finish(ppr_ctx* h, const char* where) {
-    cudaError_t e = cudaMemcpyAsync(h->h_ctl, h->d_ctl, sizeof(DevCtl), cudaMemcpyDeviceToHost, h->st);
+    cudaError_t e = cudaMemcpyAsync(h->h_ctl, &h->d_ctl->st, sizeof(DevStats), cudaMemcpyDeviceToHost, h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, where);
     e = cudaStreamSynchronize(h->st);
     if (e == cudaSuccess) e = cudaGetLastError();
@@ -446,7 +446,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
               dalloc(h, &h->vb.part, scan_parts(h->n) + 1) == cudaSuccess &&
               dalloc(h, &h->vb.big, h->n) == cudaSuccess &&
               dalloc(h, &h->vb.touched, h->n) == cudaSuccess &&
-              cudaMallocHost(&h->h_ctl, sizeof(DevCtl)) == cudaSuccess;
+              cudaMallocHost(&h->h_ctl, sizeof(DevStats)) == cudaSuccess;
     uint32_t *d_src = nullptr, *d_dst = nullptr;
     ok = ok && dalloc(h, &d_src, g->m) == cudaSuccess && dalloc(h, &d_dst, g->m) == cudaSuccess;
     if (!ok) {
@@ -474,7 +474,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     DevGraph dg = graph_of(h);
     launch_build_count(d_src, d_dst, g->m, h->undirected, dg, h->n, st, &launches);
     launch_caps_from_len(dg, h->vb, h->slack, h->min_cap, st, &launches);
-    unsigned long long* d_total = &h->d_ctl->pool_top;
+    unsigned long long* d_total = &h->d_ctl->st.pool_top;
     exclusive_scan_u32(h->vb.newcap, h->vb.newoff, h->n, h->vb.part, d_total, st, &launches);
     unsigned long long total = 0;
     cudaMemcpyAsync(&total, d_total, sizeof total, cudaMemcpyDeviceToHost, st);
@@ -621,8 +621,8 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     const uint64_t* kv = b.kv[wv];
     const uint64_t* ku = b.ku[wu];
     cudaMemsetAsync(b.claim, 0, sizeof(uint32_t) * N, st);
-    launch_heads(kv, b.ov[wv], N, b.rnv, b.vheads, &h->d_ctl->n_vheads, st, &launches);
-    launch_heads(ku, b.ou[wu], N, b.rnu, b.uheads, &h->d_ctl->n_uheads, st, &launches);
+    launch_heads(kv, b.ov[wv], N, b.rnv, b.vheads, &h->d_ctl->st.n_vheads, st, &launches);
+    launch_heads(ku, b.ou[wu], N, b.rnu, b.uheads, &h->d_ctl->st.n_uheads, st, &launches);
     // a1: graph store
     launch_store_validate(dg, kv, N, b, h->vb, h->d_ctl, h->force_rebuild ? 1 : 0, st, &launches);
     launch_store_apply(dg, kv, N, b, h->d_ctl, st, &launches);
@@ -637,7 +637,7 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     if (h->push_enabled) {
         PushArgs a = push_args(h);
         a.seed_v = h->vb.touched;
-        a.n_seed_v_dev = &h->d_ctl->n_touched;
+        a.n_seed_v_dev = &h->d_ctl->st.n_touched;
         rs = run_push(h, a, &launches);
         if (rs != PPR_OK) return rs;
     }
@@ -738,7 +738,7 @@ ppr_status ppr_export_edges(ppr_ctx* h, uint32_t* src_out, uint32_t* dst_out, ui
         cudaStream_t st = h->st;
         DevGraph dg = graph_of(h);
         launch_len_to_u32(dg, lens, st, &launches);
-        exclusive_scan_u32(lens, off, h->n, h->vb.part, &h->d_ctl->pool_top, st, &launches);
+        exclusive_scan_u32(lens, off, h->n, h->vb.part, &h->d_ctl->st.pool_top, st, &launches);
         launch_export(dg, (int)h->active, off, k[0], st, &launches);
         cudaMemsetAsync(v[0], 0, sizeof(uint32_t) * m, st);
         int w = radix_sort_pairs(k[0], v[0], k[1], v[1], m, h->shifts, h->npasses, hist, st,

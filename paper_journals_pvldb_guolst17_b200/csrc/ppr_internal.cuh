@@ -25,31 +25,42 @@ struct __align__(16) Slab {
 // error codes written by kernels into DevCtl::err (mirror ppr_status)
 enum : int { KERR_OK = 0, KERR_RANGE = -2, KERR_NOENT = -3, KERR_NOCONV = -7, KERR_OVERFLOW = -8 };
 
-struct DevCtl {
-    // frontier counters / tile counters, triple-buffered by iteration (push.cu)
-    unsigned long long fcount[3];
-    unsigned long long tilectr[3];
-    // grid barrier
-    unsigned int bar_count;
-    unsigned int bar_gen;
-    // push statistics
+// Statistics and flags the host reads back after every call (one D2H copy).
+struct DevStats {
     unsigned long long pushes;
     unsigned long long pushed_edges;
     unsigned long long max_frontier;
     unsigned int iters[2];     // [0] = POS, [1] = NEG
-    // batch pipeline
     int err;                   // KERR_*
     int rebuild;               // 1: the store takes the rebuild path this batch
     unsigned int active_pool;  // index of the active slab pool
     unsigned int n_vheads;     // v-segments in the (v,u)-sorted batch
     unsigned int n_uheads;     // u-segments in the (u,v)-sorted batch
     unsigned int n_touched;    // distinct u restored
-    unsigned long long pool_top; // entries used in the active pool (after rebuild)
-    unsigned long long dup_enqueue; // debug: enqueues of an entry already queued
+    unsigned long long pool_top; // scan total (rebuild / build)
     long long arc_delta;       // net change of the arc count this batch
     unsigned int n_big;        // vertices copied warp-wide in a rebuild
     unsigned int pad0;
-    unsigned long long pad[2];
+};
+
+// A counter alone on its 128-byte line: the per-round counters, the tile
+// claims and the grid barrier are hammered by every CTA, so none of them
+// may share a line with another.
+struct __align__(128) HotU64 {
+    unsigned long long v;
+    unsigned long long pad[15];
+};
+struct __align__(128) HotU32 {
+    unsigned int v;
+    unsigned int pad[31];
+};
+
+struct DevCtl {
+    HotU64 fcount[3];   // frontier counters, triple-buffered by round (push.cu)
+    HotU64 tilectr[3];  // tile claims, triple-buffered by round
+    HotU32 bar_count;   // grid barrier arrivals
+    HotU32 bar_gen;     // grid barrier generation
+    DevStats st;
 };
 
 struct DevGraph {
@@ -93,15 +104,15 @@ __device__ __forceinline__ void st_release_u32(unsigned int* p, unsigned int v) 
 __device__ __forceinline__ void grid_sync(DevCtl* ctl) {
     __syncthreads();
     if (threadIdx.x == 0) {
-        unsigned int gen = ld_acquire_u32(&ctl->bar_gen);
+        unsigned int gen = ld_acquire_u32(&ctl->bar_gen.v);
         __threadfence();
-        unsigned int arrived = atomicAdd(&ctl->bar_count, 1u) + 1u;
+        unsigned int arrived = atomicAdd(&ctl->bar_count.v, 1u) + 1u;
         if (arrived == gridDim.x) {
-            ctl->bar_count = 0;
+            ctl->bar_count.v = 0;
             __threadfence();
-            st_release_u32(&ctl->bar_gen, gen + 1u);
+            st_release_u32(&ctl->bar_gen.v, gen + 1u);
         } else {
-            while (ld_acquire_u32(&ctl->bar_gen) == gen) __nanosleep(20);
+            while (ld_acquire_u32(&ctl->bar_gen.v) == gen) __nanosleep(32);
         }
         __threadfence();
     }

@@ -60,6 +60,7 @@ struct Smem {
     unsigned int wq[NW];                  // slice fill at the end-of-round flush
     unsigned long long gbase;
     unsigned long long next;              // next claimed tile
+    unsigned long long cround;            // this round's frontier size
     uint32_t warp_tmp[NW + 1];            // block-scan scratch
 };
 
@@ -174,6 +175,15 @@ __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
         r = valid ? __ldcg(&a.W[idx]) : 0.0;   // Alg 3: the snapshot S
         push = valid;
     }
+    // Alg 4 lines 20-21, fused and issued before the edge walk so its latency
+    // overlaps it: R(u) -= r_u atomically (its result decides the re-enqueue,
+    // DESIGN.md K-PUSH) and P(u) += a r_u as a fire-and-forget reduction (one
+    // entry per vertex per round, so no contention).
+    double self_old = 0.0;
+    if (KIND == K_OPT && push) {
+        self_old = atomicAdd(ru, -r);
+        atomicAdd(a.g.P + (size_t)sidx * n + u, __dmul_rn(alpha, r));
+    }
     uint32_t len = 0;
     unsigned long long off = 0;
     if (push) {
@@ -193,13 +203,14 @@ __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
         c.edges += E;
         if (c.trace_edges && E) atomicAdd(c.trace_edges, (unsigned long long)E);
     }
-    for (uint32_t rb = w * 32 * U; rb < E; rb += NW * 32 * U) {
+    // 32-edge chunks dealt round-robin to the warps (chunk w + NW*i), U per step
+    for (uint32_t cb = w; cb * 32 < E; cb += NW * U) {
         ensure_room(s, c, 32 * U);
         uint32_t v[U];
         int j[U];
 #pragma unroll
         for (int k = 0; k < U; k++) {
-            const uint32_t e = rb + 32 * k + L;
+            const uint32_t e = (cb + NW * k) * 32 + L;
             j[k] = -1;
             v[k] = 0;
             if (e < E) {
@@ -229,14 +240,10 @@ __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
             warp_enqueue(s, c, enq, ev);
         }
     }
-    if (KIND == K_OPT) {  // Alg 4 lines 20-23, fused: atomic subtract, re-enqueue on its result
+    if (KIND == K_OPT) {  // re-enqueue on the result of the fused self-update
         bool re = false;
         if (push) {
-            const double old = atomicAdd(ru, -r);
-            const double cur = __dadd_rn(old, -r);
-            double* pu = a.g.P + (size_t)sidx * n + u;
-            __stcg(pu, __dadd_rn(__ldcg(pu), __dmul_rn(alpha, r)));
-            re = push_cond<POS>(cur, eps);
+            re = push_cond<POS>(__dadd_rn(self_old, -r), eps);
             c.pushes++;
         }
         ensure_room(s, c, 32);
@@ -259,6 +266,7 @@ __device__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a, const unsigned
     uint64_t t = blockIdx.x;
     while (t < ntiles) {
         cta_tile<POS, KIND>(s, c, a, Fin, C, t * T, T, top);
+        if (ntiles <= gridDim.x) break;  // every tile was assigned statically
         if (threadIdx.x == 0) s.next = atomicAdd(tc, 1ull) + gridDim.x;
         __syncthreads();
         t = s.next;
@@ -368,33 +376,36 @@ __device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
     const int ph = POS ? 0 : 1;
     // seed into F[it%2] / fcount[it%3]; both that and the next counter are 0 here
     c.Fout = a.F[it & 1];
-    c.cnt_out = &ctl->fcount[it % 3];
+    c.cnt_out = &ctl->fcount[it % 3].v;
     seed_phase<POS>(s, c, a);
     block_flush(s, c);
     grid_sync(ctl);
     uint32_t pit = 0;
     uint64_t C = 0;
     while (true) {
-        C = *(volatile unsigned long long*)&ctl->fcount[it % 3];
+        // one load per CTA (grid_sync ended with __syncthreads)
+        if (threadIdx.x == 0) s.cround = *(volatile unsigned long long*)&ctl->fcount[it % 3].v;
+        __syncthreads();
+        C = s.cround;
         c.trace_edges = (a.trace && it < a.trace_cap) ? &a.trace[4ull * it + 2] : nullptr;
         if (blockIdx.x == 0 && threadIdx.x == 0) {
             if (c.trace_edges) {
                 a.trace[4ull * it] = C | ((unsigned long long)ph << 63);
                 a.trace[4ull * it + 1] = global_ns();
             }
-            ctl->fcount[(it + 2) % 3] = 0;
-            ctl->tilectr[(it + 2) % 3] = 0;
+            ctl->fcount[(it + 2) % 3].v = 0;
+            ctl->tilectr[(it + 2) % 3].v = 0;
             if (C > 0 && !(a.max_iters && pit >= a.max_iters)) {
-                ctl->iters[ph]++;
-                atomicMax(&ctl->max_frontier, (unsigned long long)C);
+                ctl->st.iters[ph]++;
+                atomicMax(&ctl->st.max_frontier, (unsigned long long)C);
             }
-            if (C > 0 && pit >= a.iter_cap) atomicCAS(&ctl->err, KERR_OK, KERR_NOCONV);
+            if (C > 0 && pit >= a.iter_cap) atomicCAS(&ctl->st.err, KERR_OK, KERR_NOCONV);
         }
         if (C == 0 || (a.max_iters && pit >= a.max_iters) || pit >= a.iter_cap) break;
         const unsigned long long* Fin = a.F[it & 1];
         c.Fout = a.F[(it + 1) & 1];
-        c.cnt_out = &ctl->fcount[(it + 1) % 3];
-        unsigned long long* tc = &ctl->tilectr[it % 3];
+        c.cnt_out = &ctl->fcount[(it + 1) % 3].v;
+        unsigned long long* tc = &ctl->tilectr[it % 3].v;
         if (MODE == M_OPT) {
             propagate_all<POS, K_OPT>(s, c, a, Fin, C, tc);
         } else if (MODE == M_VAN || MODE == M_DUP) {
@@ -421,24 +432,24 @@ __device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
     // leave the counters of the next phase's seed round at zero
     grid_sync(ctl);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
-        ctl->fcount[0] = ctl->fcount[1] = ctl->fcount[2] = 0;
-        ctl->tilectr[0] = ctl->tilectr[1] = ctl->tilectr[2] = 0;
+        ctl->fcount[0].v = ctl->fcount[1].v = ctl->fcount[2].v = 0;
+        ctl->tilectr[0].v = ctl->tilectr[1].v = ctl->tilectr[2].v = 0;
     }
     grid_sync(ctl);
 }
 
 template <int MODE>
-__global__ void __launch_bounds__(PT, 2) k_push(const __grid_constant__ PushArgs a) {
+__global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_constant__ PushArgs a) {
     __shared__ Smem s;
     Ctx c;
     c.trace_edges = nullptr;
     c.qn = 0;
     c.pushes = 0;
     c.edges = 0;
-    if (*(volatile int*)&a.ctl->err != KERR_OK) return;  // earlier stage failed: uniform exit
-    c.pool = *(volatile unsigned*)&a.ctl->active_pool ? a.g.pool[1] : a.g.pool[0];
+    if (*(volatile int*)&a.ctl->st.err != KERR_OK) return;  // earlier stage failed: uniform exit
+    c.pool = *(volatile unsigned*)&a.ctl->st.active_pool ? a.g.pool[1] : a.g.pool[0];
     if (blockIdx.x == 0 && threadIdx.x == 0) {
-        for (int i = 0; i < 3; i++) a.ctl->fcount[i] = a.ctl->tilectr[i] = 0;
+        for (int i = 0; i < 3; i++) a.ctl->fcount[i].v = a.ctl->tilectr[i].v = 0;
     }
     grid_sync(a.ctl);
     unsigned it = 0;
@@ -456,8 +467,8 @@ __global__ void __launch_bounds__(PT, 2) k_push(const __grid_constant__ PushArgs
     if (c.edges) atomicAdd(&s_red[1], c.edges);
     __syncthreads();
     if (threadIdx.x == 0) {
-        if (s_red[0]) atomicAdd(&a.ctl->pushes, s_red[0]);
-        if (s_red[1]) atomicAdd(&a.ctl->pushed_edges, s_red[1]);
+        if (s_red[0]) atomicAdd(&a.ctl->st.pushes, s_red[0]);
+        if (s_red[1]) atomicAdd(&a.ctl->st.pushed_edges, s_red[1]);
     }
 }
 
@@ -469,7 +480,7 @@ cudaError_t launch_mode(const PushArgs& a, int num_sms, cudaStream_t st) {
             cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push<MODE>, PT, 0);
         if (e != cudaSuccess) return e;
         if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
-        if (blocks_per_sm > 2) blocks_per_sm = 2;
+        if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
     }
     dim3 grid(num_sms * blocks_per_sm), block(PT);
     PushArgs copy = a;

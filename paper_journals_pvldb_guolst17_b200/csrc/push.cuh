@@ -7,8 +7,8 @@
 
 namespace ppr {
 
-constexpr int PUSH_THREADS = 512;   // one frontier tile = PUSH_THREADS entries
-constexpr int PUSH_QCAP = 4096;     // per-CTA shared-memory enqueue buffer (u64 entries)
+constexpr int PUSH_THREADS = 256;   // one frontier tile = up to PUSH_THREADS entries
+constexpr int PUSH_MIN_BLOCKS = 4;  // resident CTAs per SM (persistent grid = SMs x this)
 
 struct PushArgs {
     DevGraph g;

@@ -24,7 +24,7 @@ namespace ppr {
 
 namespace {
 
-__device__ __forceinline__ void set_err(DevCtl* ctl, int code) { atomicCAS(&ctl->err, KERR_OK, code); }
+__device__ __forceinline__ void set_err(DevCtl* ctl, int code) { atomicCAS(&ctl->st.err, KERR_OK, code); }
 
 __device__ __forceinline__ uint32_t warp_sum_u32(uint32_t x) {
 #pragma unroll
@@ -88,14 +88,13 @@ __device__ __forceinline__ bool is_run_head(const uint64_t* keys, uint64_t j, ui
 // ---------------------------------------------------------------- a0 keys
 
 __global__ void k_ctl_reset(DevCtl* ctl) {
-    ctl->pushes = ctl->pushed_edges = ctl->max_frontier = 0;
-    ctl->iters[0] = ctl->iters[1] = 0;
-    ctl->err = KERR_OK;
-    ctl->rebuild = 0;
-    ctl->n_vheads = ctl->n_uheads = ctl->n_touched = 0;
-    ctl->dup_enqueue = 0;
-    ctl->arc_delta = 0;
-    ctl->n_big = 0;
+    ctl->st.pushes = ctl->st.pushed_edges = ctl->st.max_frontier = 0;
+    ctl->st.iters[0] = ctl->st.iters[1] = 0;
+    ctl->st.err = KERR_OK;
+    ctl->st.rebuild = 0;
+    ctl->st.n_vheads = ctl->st.n_uheads = ctl->st.n_touched = 0;
+    ctl->st.arc_delta = 0;
+    ctl->st.n_big = 0;
 }
 
 __global__ void k_batch_keys(const uint32_t* __restrict__ is, const uint32_t* __restrict__ id,
@@ -164,11 +163,11 @@ __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, ui
                                  BatchBufs b, uint32_t* __restrict__ vseg, DevCtl* ctl,
                                  int force_rebuild) {
     const unsigned lane = threadIdx.x & 31u;
-    const uint32_t nseg = *(volatile unsigned*)&ctl->n_vheads;
-    const uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->active_pool];
+    const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
+    const uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->st.active_pool];
     const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
-    if (force_rebuild && blockIdx.x == 0 && threadIdx.x == 0) ctl->rebuild = 1;
+    if (force_rebuild && blockIdx.x == 0 && threadIdx.x == 0) ctl->st.rebuild = 1;
     for (uint64_t w = warp; w < nseg; w += nwarps) {
         const uint64_t i0 = b.vheads[w];
         const uint32_t v = (uint32_t)(kv[i0] >> 32);
@@ -208,8 +207,8 @@ __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, ui
             b.seg_I[i0] = I;
             vseg[v] = (uint32_t)i0;
             if (found < Dn) set_err(ctl, KERR_NOENT);  // deletion of an absent arc
-            if ((uint64_t)sl.len - found + I > sl.cap) ctl->rebuild = 1;
-            atomicAdd((unsigned long long*)&ctl->arc_delta,
+            if ((uint64_t)sl.len - found + I > sl.cap) ctl->st.rebuild = 1;
+            atomicAdd((unsigned long long*)&ctl->st.arc_delta,
                       (unsigned long long)((long long)I - (long long)Dn));
         }
     }
@@ -217,10 +216,10 @@ __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, ui
 
 __global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, BatchBufs b,
                               DevCtl* ctl) {
-    if (*(volatile int*)&ctl->err != KERR_OK || *(volatile int*)&ctl->rebuild) return;
+    if (*(volatile int*)&ctl->st.err != KERR_OK || *(volatile int*)&ctl->st.rebuild) return;
     const unsigned lane = threadIdx.x & 31u;
-    const uint32_t nseg = *(volatile unsigned*)&ctl->n_vheads;
-    uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->active_pool];
+    const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
+    uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->st.active_pool];
     const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     for (uint64_t w = warp; w < nseg; w += nwarps) {
@@ -269,7 +268,7 @@ __global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, Batch
 
 __global__ void k_rebuild_caps(DevGraph g, BatchBufs b, VertexBufs vb, double slack,
                                uint32_t min_cap, DevCtl* ctl) {
-    if (*(volatile int*)&ctl->err != KERR_OK || !*(volatile int*)&ctl->rebuild) return;
+    if (*(volatile int*)&ctl->st.err != KERR_OK || !*(volatile int*)&ctl->st.rebuild) return;
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x) {
         uint32_t len = g.slab[v].len;
@@ -281,8 +280,8 @@ __global__ void k_rebuild_caps(DevGraph g, BatchBufs b, VertexBufs vb, double sl
 }
 
 __global__ void k_rebuild_copy_small(DevGraph g, VertexBufs vb, uint64_t alt_cap, DevCtl* ctl) {
-    if (*(volatile int*)&ctl->err != KERR_OK || !*(volatile int*)&ctl->rebuild) return;
-    const unsigned act = *(volatile unsigned*)&ctl->active_pool;
+    if (*(volatile int*)&ctl->st.err != KERR_OK || !*(volatile int*)&ctl->st.rebuild) return;
+    const unsigned act = *(volatile unsigned*)&ctl->st.active_pool;
     const uint32_t* src = g.pool[act];
     uint32_t* dst = g.pool[act ^ 1u];
     const unsigned lane = threadIdx.x & 31u;
@@ -308,7 +307,7 @@ __global__ void k_rebuild_copy_small(DevGraph g, VertexBufs vb, uint64_t alt_cap
         const unsigned m = __ballot_sync(0xffffffffu, big);
         if (m) {
             unsigned base = 0;
-            if (lane == 0) base = atomicAdd(&ctl->n_big, (unsigned)__popc(m));
+            if (lane == 0) base = atomicAdd(&ctl->st.n_big, (unsigned)__popc(m));
             base = __shfl_sync(0xffffffffu, base, 0);
             if (big) vb.big[base + __popc(m & ((1u << lane) - 1u))] = (uint32_t)v;
         }
@@ -317,12 +316,12 @@ __global__ void k_rebuild_copy_small(DevGraph g, VertexBufs vb, uint64_t alt_cap
 
 __global__ void k_rebuild_copy_big(DevGraph g, const uint64_t* __restrict__ kv, BatchBufs b,
                                    VertexBufs vb, uint64_t alt_cap, DevCtl* ctl) {
-    if (*(volatile int*)&ctl->err != KERR_OK || !*(volatile int*)&ctl->rebuild) return;
+    if (*(volatile int*)&ctl->st.err != KERR_OK || !*(volatile int*)&ctl->st.rebuild) return;
     const unsigned lane = threadIdx.x & 31u;
-    const unsigned act = *(volatile unsigned*)&ctl->active_pool;
+    const unsigned act = *(volatile unsigned*)&ctl->st.active_pool;
     const uint32_t* src = g.pool[act];
     uint32_t* dst = g.pool[act ^ 1u];
-    const uint32_t nbig = *(volatile unsigned*)&ctl->n_big;
+    const uint32_t nbig = *(volatile unsigned*)&ctl->st.n_big;
     const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     for (uint64_t w = warp; w < nbig; w += nwarps) {
@@ -373,13 +372,13 @@ __global__ void k_rebuild_copy_big(DevGraph g, const uint64_t* __restrict__ kv, 
 }
 
 __global__ void k_rebuild_finish(DevCtl* ctl) {
-    if (ctl->err != KERR_OK || !ctl->rebuild) return;
-    ctl->active_pool ^= 1u;
+    if (ctl->st.err != KERR_OK || !ctl->st.rebuild) return;
+    ctl->st.active_pool ^= 1u;
 }
 
 __global__ void k_seg_cleanup(const uint64_t* __restrict__ kv, BatchBufs b,
                               uint32_t* __restrict__ vseg, DevCtl* ctl) {
-    const uint32_t nseg = *(volatile unsigned*)&ctl->n_vheads;
+    const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
     for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nseg;
          w += (uint64_t)gridDim.x * blockDim.x)
         vseg[kv[b.vheads[w]] >> 32] = NONE;
@@ -389,8 +388,8 @@ __global__ void k_seg_cleanup(const uint64_t* __restrict__ kv, BatchBufs b,
 
 __global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t N, BatchBufs b,
                           uint32_t* __restrict__ touched, DevCtl* ctl) {
-    if (*(volatile int*)&ctl->err != KERR_OK) return;
-    const uint32_t nseg = *(volatile unsigned*)&ctl->n_uheads;
+    if (*(volatile int*)&ctl->st.err != KERR_OK) return;
+    const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_uheads;
     const double a = g.alpha;
     for (uint64_t k = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; k < nseg;
          k += (uint64_t)gridDim.x * blockDim.x) {
@@ -428,7 +427,7 @@ __global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t 
                 r = one - pu / a;  // Eq. 2 with an empty sum (reading R4)
             g.R[base + u] = r;
         }
-        const unsigned pos = atomicAdd(&ctl->n_touched, 1u);
+        const unsigned pos = atomicAdd(&ctl->st.n_touched, 1u);
         touched[pos] = u;
     }
 }
@@ -558,7 +557,7 @@ void launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, con
     (void)N;
     k_rebuild_caps<<<grid_for(g.n, 256), 256, 0, st>>>(g, b, vb, sp.slack, sp.min_cap, ctl);
     ++*launches;
-    exclusive_scan_u32(vb.newcap, vb.newoff, g.n, vb.part, &ctl->pool_top, st, launches);
+    exclusive_scan_u32(vb.newcap, vb.newoff, g.n, vb.part, &ctl->st.pool_top, st, launches);
     k_rebuild_copy_small<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb, sp.alt_cap, ctl);
     k_rebuild_copy_big<<<148 * 8, 256, 0, st>>>(g, kv, b, vb, sp.alt_cap, ctl);
     k_rebuild_finish<<<1, 1, 0, st>>>(ctl);

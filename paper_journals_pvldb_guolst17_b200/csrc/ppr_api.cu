@@ -327,7 +327,7 @@ void destroy_all(ppr_ctx* h) {
     dfree(h, h->vb.vseg, h->n);
     dfree(h, h->vb.newcap, h->n);
     dfree(h, h->vb.newoff, h->n);
-    dfree(h, h->vb.part, scan_parts(h->n) + 1);
+    dfree(h, h->vb.part, std::max<uint64_t>(scan_parts(h->n) + 1, 8192));
     dfree(h, h->vb.big, h->n);
     dfree(h, h->vb.touched, h->n);
     if (h->h_ctl) cudaFreeHost(h->h_ctl);
@@ -443,7 +443,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
               dalloc(h, &h->d_ctl, 1) == cudaSuccess && dalloc(h, &h->vb.vseg, h->n) == cudaSuccess &&
               dalloc(h, &h->vb.newcap, h->n) == cudaSuccess &&
               dalloc(h, &h->vb.newoff, h->n) == cudaSuccess &&
-              dalloc(h, &h->vb.part, scan_parts(h->n) + 1) == cudaSuccess &&
+              dalloc(h, &h->vb.part, std::max<uint64_t>(scan_parts(h->n) + 1, 8192)) == cudaSuccess &&
               dalloc(h, &h->vb.big, h->n) == cudaSuccess &&
               dalloc(h, &h->vb.touched, h->n) == cudaSuccess &&
               cudaMallocHost(&h->h_ctl, sizeof(DevStats)) == cudaSuccess;

@@ -9,6 +9,8 @@
 //               __match_any_sync / popc per warp and per-warp digit offsets in
 //               shared memory, then a scatter to
 //               digit_base + tile_offset + rank.
+// Small sorts (n <= 2^18) use 512-key tiles and, with at most 64 tiles,
+// fold the offset scan into the scatter (two kernels per pass).
 // Keys are read striped (item r of thread t is tile_base + r*256 + t) so
 // loads are coalesced and the (round, thread) order is the input order,
 // which keeps the sort stable.
@@ -19,6 +21,7 @@ namespace ppr {
 
 // ---------------------------------------------------------------- radix sort
 
+template <int ITEMS>
 __global__ void __launch_bounds__(RS_THREADS) k_rs_hist(const uint64_t* __restrict__ keys,
                                                         uint64_t n, int shift,
                                                         uint32_t* __restrict__ hist,
@@ -26,9 +29,9 @@ __global__ void __launch_bounds__(RS_THREADS) k_rs_hist(const uint64_t* __restri
     __shared__ uint32_t s_h[256];
     s_h[threadIdx.x] = 0;
     __syncthreads();
-    const uint64_t base = (uint64_t)blockIdx.x * RS_TILE;
-#pragma unroll 4
-    for (int r = 0; r < RS_ITEMS; r++) {
+    const uint64_t base = (uint64_t)blockIdx.x * RS_THREADS * ITEMS;
+#pragma unroll
+    for (int r = 0; r < ITEMS; r++) {
         uint64_t i = base + (uint64_t)r * RS_THREADS + threadIdx.x;
         if (i < n) atomicAdd(&s_h[(keys[i] >> shift) & 255u], 1u);
     }
@@ -54,6 +57,9 @@ __global__ void __launch_bounds__(RS_THREADS) k_rs_scan(uint32_t* __restrict__ h
     if (threadIdx.x == 0) hist[(uint64_t)256 * ntiles + d] = carry;
 }
 
+// FUSED: the tile offsets are summed here from the raw per-tile counts
+// (ntiles <= RS_FUSED_MAX_TILES), otherwise k_rs_scan has prepared them.
+template <int ITEMS, bool FUSED>
 __global__ void __launch_bounds__(RS_THREADS) k_rs_scatter(
     const uint64_t* __restrict__ kin, const uint32_t* __restrict__ vin,
     uint64_t* __restrict__ kout, uint32_t* __restrict__ vout, uint64_t n, int shift,
@@ -64,15 +70,27 @@ __global__ void __launch_bounds__(RS_THREADS) k_rs_scatter(
     __shared__ uint32_t s_wc[NW][256];   // per-warp digit counts this round
     __shared__ uint32_t s_wo[NW][256];   // per-warp digit offsets this round
     const unsigned t = threadIdx.x, lane = t & 31u, warp = t >> 5;
+    uint32_t tot_t, pre_t;
+    if (FUSED) {
+        const uint32_t* row = hist + (uint64_t)t * ntiles;
+        tot_t = pre_t = 0;
+        for (uint32_t b = 0; b < ntiles; b++) {
+            const uint32_t x = row[b];
+            tot_t += x;
+            pre_t += b < blockIdx.x ? x : 0u;
+        }
+    } else {
+        tot_t = hist[(uint64_t)256 * ntiles + t];
+        pre_t = hist[(uint64_t)t * ntiles + blockIdx.x];
+    }
     // digit base = exclusive scan of digit totals (thread t owns digit t)
-    uint32_t tot_t = hist[(uint64_t)256 * ntiles + t];
     uint32_t dbase = block_exclusive_scan_u32<RS_THREADS>(tot_t, s_warp, nullptr);
-    s_run[t] = dbase + hist[(uint64_t)t * ntiles + blockIdx.x];
+    s_run[t] = dbase + pre_t;
 #pragma unroll
     for (int w = 0; w < NW; w++) s_wc[w][t] = 0;
     __syncthreads();
-    const uint64_t base = (uint64_t)blockIdx.x * RS_TILE;
-    for (int r = 0; r < RS_ITEMS; r++) {
+    const uint64_t base = (uint64_t)blockIdx.x * RS_THREADS * ITEMS;
+    for (int r = 0; r < ITEMS; r++) {
         uint64_t i = base + (uint64_t)r * RS_THREADS + t;
         bool valid = i < n;
         uint64_t k = valid ? kin[i] : 0ull;
@@ -106,15 +124,32 @@ int radix_sort_pairs(uint64_t* k0, uint32_t* v0, uint64_t* k1, uint32_t* v1, uin
                      const int* shifts, int npasses, uint32_t* hist, cudaStream_t st,
                      uint32_t* launches) {
     if (n <= 1 || npasses == 0) return 0;
-    uint32_t ntiles = (uint32_t)rs_tiles(n);
+    const uint32_t ntiles = (uint32_t)rs_tiles(n);
+    const bool small = rs_items(n) == 2;
+    const bool fused = ntiles <= RS_FUSED_MAX_TILES;
     uint64_t *ki = k0, *ko = k1;
     uint32_t *vi = v0, *vo = v1;
     int where = 0;
     for (int p = 0; p < npasses; p++) {
-        k_rs_hist<<<ntiles, RS_THREADS, 0, st>>>(ki, n, shifts[p], hist, ntiles);
-        k_rs_scan<<<256, RS_THREADS, 0, st>>>(hist, ntiles);
-        k_rs_scatter<<<ntiles, RS_THREADS, 0, st>>>(ki, vi, ko, vo, n, shifts[p], hist, ntiles);
-        *launches += 3;
+        if (small) {
+            k_rs_hist<2><<<ntiles, RS_THREADS, 0, st>>>(ki, n, shifts[p], hist, ntiles);
+            if (fused) {
+                k_rs_scatter<2, true><<<ntiles, RS_THREADS, 0, st>>>(ki, vi, ko, vo, n, shifts[p],
+                                                                     hist, ntiles);
+            } else {
+                k_rs_scan<<<256, RS_THREADS, 0, st>>>(hist, ntiles);
+                k_rs_scatter<2, false><<<ntiles, RS_THREADS, 0, st>>>(ki, vi, ko, vo, n,
+                                                                      shifts[p], hist, ntiles);
+                ++*launches;
+            }
+        } else {
+            k_rs_hist<16><<<ntiles, RS_THREADS, 0, st>>>(ki, n, shifts[p], hist, ntiles);
+            k_rs_scan<<<256, RS_THREADS, 0, st>>>(hist, ntiles);
+            k_rs_scatter<16, false><<<ntiles, RS_THREADS, 0, st>>>(ki, vi, ko, vo, n, shifts[p],
+                                                                   hist, ntiles);
+            ++*launches;
+        }
+        *launches += 2;
         uint64_t* tk = ki;
         ki = ko;
         ko = tk;

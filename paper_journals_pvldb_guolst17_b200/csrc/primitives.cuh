@@ -8,12 +8,20 @@
 namespace ppr {
 
 constexpr int RS_THREADS = 256;
-constexpr int RS_ITEMS = 16;
-constexpr int RS_TILE = RS_THREADS * RS_ITEMS;  // keys per CTA per pass
-
-inline uint64_t rs_tiles(uint64_t n) { return (n + RS_TILE - 1) / RS_TILE; }
+// keys per thread per pass: small batches use short tiles so that many CTAs
+// share a pass, large ones long tiles so that the per-tile histograms stay few
+inline int rs_items(uint64_t n) { return n <= (1u << 18) ? 2 : 16; }
+inline uint64_t rs_tiles(uint64_t n) {
+    const uint64_t tile = (uint64_t)RS_THREADS * rs_items(n);
+    return (n + tile - 1) / tile;
+}
+constexpr uint32_t RS_FUSED_MAX_TILES = 64;  // at most this many tiles: no separate scan kernel
 // scratch entries (u32) the sort needs for n keys
-inline uint64_t rs_hist_entries(uint64_t n) { return 256 * (rs_tiles(n) + 1) + 256; }
+// (valid for every sort of m <= n keys)
+inline uint64_t rs_hist_entries(uint64_t n) {
+    uint64_t t = rs_tiles(n), ts = rs_tiles(n < (1u << 18) ? n : (1u << 18));
+    return 256 * ((t > ts ? t : ts) + 1) + 256;
+}
 
 // Sorts n pairs by the bits [shift, shift+8) for every shift in `shifts`
 // (stable LSD).  Data ping-pongs between (k0,v0) and (k1,v1); returns 0 if

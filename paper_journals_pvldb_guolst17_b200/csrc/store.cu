@@ -17,6 +17,7 @@
 //                d_k = 0 gives R(u) = 1[u=s] - P(u)/a (reading R4).
 // Identical (u, v) updates are first reduced to their net multiplicity so an
 // insertion and a deletion of the same arc in one batch cancel exactly.
+#include "block_scan.cuh"
 #include "primitives.cuh"
 #include "store.cuh"
 
@@ -265,37 +266,125 @@ __global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, Batch
 }
 
 // ---------------------------------------------------------------- a1 rebuild
+//
+// One cooperative kernel (it exits at once unless DevCtl::rebuild is set, so
+// the common no-overflow batch pays one short launch): capacities of every
+// slab with the batch merged -> exclusive scan -> stable copy of each slab
+// into the other pool with its deletions dropped and insertions appended ->
+// flip the active pool.  Phases are separated by grid barriers.
 
-__global__ void k_rebuild_caps(DevGraph g, BatchBufs b, VertexBufs vb, double slack,
-                               uint32_t min_cap, DevCtl* ctl) {
-    if (*(volatile int*)&ctl->st.err != KERR_OK || !*(volatile int*)&ctl->st.rebuild) return;
-    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
-         v += (uint64_t)gridDim.x * blockDim.x) {
-        uint32_t len = g.slab[v].len;
-        const uint32_t sg = vb.vseg[v];
-        if (sg != NONE) len = len - b.seg_D[sg] + b.seg_I[sg];
-        uint32_t extra = (uint32_t)ceil((double)len * slack);
-        vb.newcap[v] = len + (extra > min_cap ? extra : min_cap);
-    }
+constexpr int RB_THREADS = 256;
+
+// new length of v after this batch (the batch's segment for v, if any)
+__device__ __forceinline__ uint32_t merged_len(const DevGraph& g, const BatchBufs& b,
+                                               const VertexBufs& vb, uint64_t v) {
+    uint32_t len = g.slab[v].len;
+    const uint32_t sg = vb.vseg[v];
+    if (sg != NONE) len = len - b.seg_D[sg] + b.seg_I[sg];
+    return len;
 }
 
-__global__ void k_rebuild_copy_small(DevGraph g, VertexBufs vb, uint64_t alt_cap, DevCtl* ctl) {
-    if (*(volatile int*)&ctl->st.err != KERR_OK || !*(volatile int*)&ctl->st.rebuild) return;
-    const unsigned act = *(volatile unsigned*)&ctl->st.active_pool;
-    const uint32_t* src = g.pool[act];
-    uint32_t* dst = g.pool[act ^ 1u];
+__device__ __forceinline__ uint32_t cap_for(uint32_t len, double slack, uint32_t min_cap) {
+    const uint32_t extra = (uint32_t)ceil((double)len * slack);
+    return len + (extra > min_cap ? extra : min_cap);
+}
+
+// warp-wide stable copy of slab v into dst[no ..] without its claimed
+// deletions, followed by its net insertions; returns the new length
+__device__ uint32_t copy_merged_warp(const uint32_t* src, uint32_t* dst, const Slab sl,
+                                     unsigned long long no, const uint64_t* kv, const BatchBufs& b,
+                                     uint32_t sg) {
     const unsigned lane = threadIdx.x & 31u;
-    for (uint64_t b0 = (uint64_t)blockIdx.x * blockDim.x; b0 < g.n;
-         b0 += (uint64_t)gridDim.x * blockDim.x) {
-        const uint64_t v = b0 + threadIdx.x;
+    const uint32_t D = sg != NONE ? b.seg_D[sg] : 0u;
+    const uint32_t* dp = sg != NONE ? b.delpos + sg : nullptr;
+    uint32_t pos = 0;
+    for (uint32_t p0 = 0; p0 < sl.len; p0 += 32) {
+        const uint32_t p = p0 + lane;
+        const bool keep = p < sl.len && !(D && contains_u32(dp, D, p));
+        const unsigned m = __ballot_sync(0xffffffffu, keep);
+        if (keep) dst[no + pos + __popc(m & ((1u << lane) - 1u))] = src[sl.off + p];
+        pos += __popc(m);
+    }
+    if (sg != NONE) {
+        const uint64_t i0 = sg, i1 = b.seg_end[sg];
+        for (uint64_t j0 = i0; j0 < i1; j0 += 32) {
+            const uint64_t j = j0 + lane;
+            uint32_t c = 0, x = 0;
+            if (j < i1 && is_run_head(kv, j, i0)) {
+                const int32_t net = b.rnv[j];
+                if (net > 0) {
+                    c = (uint32_t)net;
+                    x = (uint32_t)kv[j];
+                }
+            }
+            uint32_t tot;
+            const uint32_t ex = warp_excl_scan_u32(c, tot);
+            for (uint32_t k = 0; k < c; k++) dst[no + pos + ex + k] = x;
+            pos += tot;
+        }
+    }
+    return pos;
+}
+
+__global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64_t* __restrict__ kv,
+                                                        BatchBufs b, VertexBufs vb, double slack,
+                                                        uint32_t min_cap, uint64_t alt_cap,
+                                                        DevCtl* ctl) {
+    if (*(volatile int*)&ctl->st.err != KERR_OK || !*(volatile int*)&ctl->st.rebuild) return;
+    __shared__ uint32_t s_warp[RB_THREADS / 32 + 1];
+    __shared__ unsigned long long s_warp64[RB_THREADS / 32 + 1];
+    const unsigned act = *(volatile unsigned*)&ctl->st.active_pool;
+    const uint32_t* src = act ? g.pool[1] : g.pool[0];
+    uint32_t* dst = act ? g.pool[0] : g.pool[1];
+    const unsigned lane = threadIdx.x & 31u;
+    // contiguous vertex range of this CTA
+    const uint64_t chunk = ((uint64_t)g.n + gridDim.x - 1) / gridDim.x;
+    const uint64_t v0 = (uint64_t)blockIdx.x * chunk;
+    const uint64_t v1 = v0 + chunk < g.n ? v0 + chunk : g.n;
+    // phase 1: capacities and the CTA's sum
+    unsigned long long mysum = 0;
+    for (uint64_t v = v0 + threadIdx.x; v < v1; v += RB_THREADS) {
+        const uint32_t nc = cap_for(merged_len(g, b, vb, v), slack, min_cap);
+        vb.newcap[v] = nc;
+        mysum += nc;
+    }
+    unsigned long long cta_sum;
+    block_exclusive_scan_u64<RB_THREADS>(mysum, s_warp64, &cta_sum);
+    if (threadIdx.x == 0) vb.part[blockIdx.x] = cta_sum;
+    grid_sync(ctl);
+    // phase 2: CTA bases (every CTA scans the partials itself)
+    unsigned long long base = 0, total = 0;
+    for (uint32_t i = threadIdx.x; i < gridDim.x; i += RB_THREADS) {
+        const unsigned long long x = __ldcg(&vb.part[i]);
+        total += x;
+        if (i < blockIdx.x) base += x;
+    }
+    {
+        unsigned long long t1, t2;
+        block_exclusive_scan_u64<RB_THREADS>(base, s_warp64, &t1);
+        block_exclusive_scan_u64<RB_THREADS>(total, s_warp64, &t2);
+        base = t1;
+        total = t2;
+    }
+    if (blockIdx.x == 0 && threadIdx.x == 0) ctl->st.pool_top = total;
+    if (total > alt_cap) {  // cannot happen: the host sizes the other pool (uniform exit)
+        if (blockIdx.x == 0 && threadIdx.x == 0) atomicCAS(&ctl->st.err, KERR_OK, KERR_OVERFLOW);
+        return;
+    }
+    // phase 3: offsets and the copy of short untouched slabs (thread per vertex);
+    // long or changed slabs go to the warp-wide list
+    for (uint64_t vb0 = v0; vb0 < v1; vb0 += RB_THREADS) {
+        const uint64_t v = vb0 + threadIdx.x;
+        const uint32_t nc = v < v1 ? vb.newcap[v] : 0u;
+        uint32_t tot;
+        const uint32_t ex = block_exclusive_scan_u32<RB_THREADS>(nc, s_warp, &tot);
         bool big = false;
-        if (v < g.n) {
+        if (v < v1) {
+            const unsigned long long no = base + ex;
+            vb.newoff[v] = no;
             const Slab sl = g.slab[v];
-            const unsigned long long no = vb.newoff[v];
-            const uint32_t nc = vb.newcap[v];
-            if (no + nc > alt_cap) set_err(ctl, KERR_OVERFLOW);
             big = vb.vseg[v] != NONE || sl.len > 16;
-            if (!big && no + nc <= alt_cap) {
+            if (!big) {
                 for (uint32_t j = 0; j < sl.len; j++) dst[no + j] = src[sl.off + j];
                 Slab ns;
                 ns.off = no;
@@ -304,76 +393,35 @@ __global__ void k_rebuild_copy_small(DevGraph g, VertexBufs vb, uint64_t alt_cap
                 g.slab[v] = ns;
             }
         }
+        base += tot;
         const unsigned m = __ballot_sync(0xffffffffu, big);
         if (m) {
-            unsigned base = 0;
-            if (lane == 0) base = atomicAdd(&ctl->st.n_big, (unsigned)__popc(m));
-            base = __shfl_sync(0xffffffffu, base, 0);
-            if (big) vb.big[base + __popc(m & ((1u << lane) - 1u))] = (uint32_t)v;
+            unsigned wb = 0;
+            if (lane == 0) wb = atomicAdd(&ctl->st.n_big, (unsigned)__popc(m));
+            wb = __shfl_sync(0xffffffffu, wb, 0);
+            if (big) vb.big[wb + __popc(m & ((1u << lane) - 1u))] = (uint32_t)v;
         }
     }
-}
-
-__global__ void k_rebuild_copy_big(DevGraph g, const uint64_t* __restrict__ kv, BatchBufs b,
-                                   VertexBufs vb, uint64_t alt_cap, DevCtl* ctl) {
-    if (*(volatile int*)&ctl->st.err != KERR_OK || !*(volatile int*)&ctl->st.rebuild) return;
-    const unsigned lane = threadIdx.x & 31u;
-    const unsigned act = *(volatile unsigned*)&ctl->st.active_pool;
-    const uint32_t* src = g.pool[act];
-    uint32_t* dst = g.pool[act ^ 1u];
+    grid_sync(ctl);
+    // phase 4: warp per long / changed slab
     const uint32_t nbig = *(volatile unsigned*)&ctl->st.n_big;
-    const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
-    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    const uint64_t warp = ((uint64_t)blockIdx.x * RB_THREADS + threadIdx.x) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * RB_THREADS) >> 5;
     for (uint64_t w = warp; w < nbig; w += nwarps) {
-        const uint32_t v = vb.big[w];
+        const uint32_t v = __ldcg(&vb.big[w]);
         const Slab sl = g.slab[v];
-        const unsigned long long no = vb.newoff[v];
-        const uint32_t nc = vb.newcap[v];
-        if (no + nc > alt_cap) continue;  // flagged by the small kernel
-        const uint32_t sg = vb.vseg[v];
-        const uint32_t D = sg != NONE ? b.seg_D[sg] : 0u;
-        const uint32_t* dp = sg != NONE ? b.delpos + sg : nullptr;
-        // stable copy of the surviving entries
-        uint32_t pos = 0;
-        for (uint32_t p0 = 0; p0 < sl.len; p0 += 32) {
-            const uint32_t p = p0 + lane;
-            const bool keep = p < sl.len && !(D && contains_u32(dp, D, p));
-            const unsigned m = __ballot_sync(0xffffffffu, keep);
-            if (keep) dst[no + pos + __popc(m & ((1u << lane) - 1u))] = src[sl.off + p];
-            pos += __popc(m);
-        }
-        // insertions
-        if (sg != NONE) {
-            const uint64_t i0 = sg, i1 = b.seg_end[sg];
-            for (uint64_t j0 = i0; j0 < i1; j0 += 32) {
-                const uint64_t j = j0 + lane;
-                uint32_t c = 0, x = 0;
-                if (j < i1 && is_run_head(kv, j, i0)) {
-                    const int32_t net = b.rnv[j];
-                    if (net > 0) {
-                        c = (uint32_t)net;
-                        x = (uint32_t)kv[j];
-                    }
-                }
-                uint32_t tot;
-                const uint32_t ex = warp_excl_scan_u32(c, tot);
-                for (uint32_t k = 0; k < c; k++) dst[no + pos + ex + k] = x;
-                pos += tot;
-            }
-        }
+        const unsigned long long no = __ldcg(&vb.newoff[v]);
+        const uint32_t len = copy_merged_warp(src, dst, sl, no, kv, b, vb.vseg[v]);
         if (lane == 0) {
             Slab ns;
             ns.off = no;
-            ns.len = pos;
-            ns.cap = nc;
+            ns.len = len;
+            ns.cap = __ldcg(&vb.newcap[v]);
             g.slab[v] = ns;
         }
     }
-}
-
-__global__ void k_rebuild_finish(DevCtl* ctl) {
-    if (ctl->st.err != KERR_OK || !ctl->st.rebuild) return;
-    ctl->st.active_pool ^= 1u;
+    grid_sync(ctl);
+    if (blockIdx.x == 0 && threadIdx.x == 0) ctl->st.active_pool = act ^ 1u;
 }
 
 __global__ void k_seg_cleanup(const uint64_t* __restrict__ kv, BatchBufs b,
@@ -555,13 +603,25 @@ void launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, con
                           const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
                           cudaStream_t st, uint32_t* launches) {
     (void)N;
-    k_rebuild_caps<<<grid_for(g.n, 256), 256, 0, st>>>(g, b, vb, sp.slack, sp.min_cap, ctl);
+    static int grid = 0;
+    if (grid == 0) {
+        int per_sm = 0, sms = 0, dev = 0;
+        cudaGetDevice(&dev);
+        cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_rebuild, RB_THREADS, 0);
+        grid = sms * (per_sm < 4 ? (per_sm < 1 ? 1 : per_sm) : 4);
+    }
+    DevGraph gg = g;
+    const uint64_t* kk = kv;
+    BatchBufs bb = b;
+    VertexBufs vv = vb;
+    double slack = sp.slack;
+    uint32_t min_cap = sp.min_cap;
+    uint64_t alt_cap = sp.alt_cap;
+    DevCtl* c = ctl;
+    void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &alt_cap, &c};
+    cudaLaunchCooperativeKernel((const void*)k_rebuild, dim3(grid), dim3(RB_THREADS), args, 0, st);
     ++*launches;
-    exclusive_scan_u32(vb.newcap, vb.newoff, g.n, vb.part, &ctl->st.pool_top, st, launches);
-    k_rebuild_copy_small<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb, sp.alt_cap, ctl);
-    k_rebuild_copy_big<<<148 * 8, 256, 0, st>>>(g, kv, b, vb, sp.alt_cap, ctl);
-    k_rebuild_finish<<<1, 1, 0, st>>>(ctl);
-    *launches += 3;
 }
 
 void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, const VertexBufs& vb,

@@ -76,6 +76,8 @@ struct ppr_ctx {
     bool poisoned = false;
     uint64_t dev_bytes = 0;
     std::vector<void*> allocs;
+    unsigned long long* d_ring = nullptr;   // PPR_MODE_ASYNC ring queue (2*S*n slots, EMPTY)
+    unsigned long long ring_cap = 0;
     unsigned long long* d_trace = nullptr;  // PPR_TRACE=1: per-round trace of the push
     uint32_t trace_cap = 0;
 };
@@ -335,11 +337,23 @@ void destroy_all(ppr_ctx* h) {
     for (auto& e : h->ev)
         if (e) cudaEventDestroy(e), e = nullptr;
     dfree(h, h->d_trace, 4ull * h->trace_cap);
+    dfree(h, h->d_ring, h->ring_cap);
     if (h->own_stream && h->st) cudaStreamDestroy(h->st);
     h->st = nullptr;
 }
 
 ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
+    if (h->mode == PPR_MODE_ASYNC && !h->d_ring) {
+        const uint64_t cap = 2ull * h->S * h->n + 1024;
+        if (dalloc(h, &h->d_ring, cap) != cudaSuccess) {
+            set_err(h, "out of device memory for the async ring (%llu slots)", (unsigned long long)cap);
+            return PPR_ENOMEM;
+        }
+        h->ring_cap = cap;
+        cudaMemsetAsync(h->d_ring, 0xFF, sizeof(unsigned long long) * cap, h->st);
+    }
+    a.ring = h->d_ring;
+    a.ring_cap = h->ring_cap;
     cudaError_t e = launch_push(h->mode, a, h->num_sms, h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, "push launch");
     ++*launches;
@@ -393,7 +407,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     o.slack = 0.25;
     o.min_cap = 4;
     if (opts) o = *opts;
-    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_VANILLA || !(o.slack >= 0.0) ||
+    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_ASYNC || !(o.slack >= 0.0) ||
         o.min_cap == 0)
         return PPR_EINVAL;
 
@@ -487,8 +501,17 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         delete h;
         return PPR_ECUDA;
     }
-    h->pool_cap[0] = total + 1024;
-    if (dalloc(h, &h->d_pool[0], h->pool_cap[0]) != cudaSuccess) {
+    // both pools get the rebuild bound with headroom up front, so steady-state
+    // batches never reallocate (ensure_alt_pool only grows them if m grows a lot)
+    {
+        const double need = std::ceil((1.0 + h->slack) * (double)arcs_in) +
+                            (double)(h->min_cap + 1) * h->n + 1024;
+        uint64_t cap = (uint64_t)(need + need / 4);
+        if (cap < total + 1024) cap = total + 1024;
+        h->pool_cap[0] = h->pool_cap[1] = cap;
+    }
+    if (dalloc(h, &h->d_pool[0], h->pool_cap[0]) != cudaSuccess ||
+        dalloc(h, &h->d_pool[1], h->pool_cap[0]) != cudaSuccess) {
         dfree(h, d_src, g->m);
         dfree(h, d_dst, g->m);
         destroy_all(h);
@@ -557,7 +580,7 @@ ppr_status ppr_set_option(ppr_ctx* h, int key, int64_t value) {
     if (h->poisoned) return PPR_EPOISONED;
     switch (key) {
         case PPR_OPT_MODE:
-            if (value < PPR_MODE_OPT || value > PPR_MODE_VANILLA) return PPR_EINVAL;
+            if (value < PPR_MODE_OPT || value > PPR_MODE_ASYNC) return PPR_EINVAL;
             h->mode = (int)value;
             return PPR_OK;
         case PPR_OPT_PUSH: h->push_enabled = value != 0; return PPR_OK;

@@ -47,7 +47,7 @@ constexpr int PT = PUSH_THREADS;
 constexpr int NW = PT / 32;     // warps per CTA
 constexpr int U = 4;            // edges per lane per step
 constexpr int QW = 256;         // per-warp queue slice (entries)
-enum { M_OPT = 0, M_EAGER = 1, M_DUP = 2, M_VAN = 3 };
+enum { M_OPT = 0, M_EAGER = 1, M_DUP = 2, M_VAN = 3, M_ASYNC = 4 };
 // how a warp tile gets r and decides enqueues
 enum { K_OPT = 0, K_EAGER = 1, K_DUP = 2, K_VAN = 3 };
 
@@ -75,6 +75,7 @@ struct Ctx {
     unsigned long long* Fout;
     unsigned long long* cnt_out;
     unsigned long long* trace_edges;  // this round's edge counter (trace mode) or null
+    unsigned long long ring_cap;      // async mode: Fout is a ring of this many slots (0: linear)
     uint32_t qn;                      // warp-uniform fill of this warp's slice
     unsigned long long pushes;        // per-thread counters
     unsigned long long edges;
@@ -83,13 +84,25 @@ struct Ctx {
 __device__ __forceinline__ unsigned lane() { return threadIdx.x & 31u; }
 __device__ __forceinline__ unsigned warp() { return threadIdx.x >> 5; }
 
+constexpr unsigned long long EMPTY = ~0ull;  // free ring slot (async mode)
+
+// writes entry e at queue position pos: a linear frontier (rounds), or a
+// ring slot (async) that must first have been freed by its consumer
+__device__ __forceinline__ void put_entry(Ctx& c, unsigned long long pos, unsigned long long e) {
+    if (c.ring_cap) {
+        pos %= c.ring_cap;
+        while (*(volatile unsigned long long*)&c.Fout[pos] != EMPTY) __nanosleep(64);
+    }
+    __stcg(&c.Fout[pos], e);
+}
+
 __device__ __forceinline__ void warp_flush(Smem& s, Ctx& c) {
     if (c.qn == 0) return;  // warp-uniform
     unsigned long long base = 0;
     if (lane() == 0) base = atomicAdd(c.cnt_out, (unsigned long long)c.qn);
     base = __shfl_sync(0xffffffffu, base, 0);
     const unsigned w = warp();
-    for (uint32_t i = lane(); i < c.qn; i += 32) c.Fout[base + i] = s.q[w][i];
+    for (uint32_t i = lane(); i < c.qn; i += 32) put_entry(c, base + i, s.q[w][i]);
     __syncwarp();
     c.qn = 0;
 }
@@ -125,7 +138,7 @@ __device__ void block_flush(Smem& s, Ctx& c) {
     }
     __syncthreads();
     const unsigned long long base = s.gbase + s.wq[w];
-    for (uint32_t i = lane(); i < c.qn; i += 32) c.Fout[base + i] = s.q[w][i];
+    for (uint32_t i = lane(); i < c.qn; i += 32) put_entry(c, base + i, s.q[w][i]);
     c.qn = 0;
     __syncthreads();
 }
@@ -150,6 +163,11 @@ __device__ __forceinline__ int owner_of(const uint32_t* scan, uint32_t e, int to
 
 // ---------------------------------------------------------------- CTA tile
 
+template <bool POS, int KIND>
+__device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
+                                          unsigned long long ent, uint64_t idx, uint32_t T,
+                                          int top);
+
 // Processes the T entries Fin[base_idx .. base_idx+T) (thread i = entry i):
 // neighbour propagation of every pushed entry and, for K_OPT, the fused
 // self-update.  Must be called by all threads of the CTA.
@@ -157,18 +175,31 @@ template <bool POS, int KIND>
 __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
                                          const unsigned long long* Fin, uint64_t C,
                                          uint64_t base_idx, uint32_t T, int top) {
-    const unsigned L = lane(), w = warp();
-    const double eps = a.g.eps, alpha = a.g.alpha;
-    const uint32_t n = a.g.n;
     const uint64_t idx = base_idx + threadIdx.x;
     const bool valid = threadIdx.x < T && idx < C;
     const unsigned long long ent = valid ? __ldcg(&Fin[idx]) : 0ull;
+    tile_body<POS, KIND>(s, c, a, valid, ent, idx, T, top);
+}
+
+// The tile's work once thread i holds entry i (valid, ent; idx indexes W).
+template <bool POS, int KIND>
+__device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
+                                          unsigned long long ent, uint64_t idx, uint32_t T,
+                                          int top) {
+    const unsigned L = lane(), w = warp();
+    const double eps = a.g.eps, alpha = a.g.alpha;
+    const uint32_t n = a.g.n;
     const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
     double* ru = a.g.R + (size_t)sidx * n + u;
     double r = 0.0;
     bool push = false;
     if (KIND == K_OPT || KIND == K_EAGER) {
         r = valid ? ld_relaxed_f64(ru) : 0.0;  // Alg 4 line 10: the current R(u)
+        // A queued vertex meets pushCond (it was enqueued on a crossing, and R(u)
+        // only grows until its own self-update).  If the relaxed load returned
+        // an older value (the async schedule has no barrier ordering it after
+        // the enqueuer's atomic), re-read at the coherence point.
+        if (KIND == K_OPT && valid && !push_cond<POS>(r, eps)) r = atomicAdd(ru, 0.0);
         push = valid && push_cond<POS>(r, eps);
         if (KIND == K_EAGER && valid) __stcg(&a.W[idx], push ? r : 0.0);
     } else {
@@ -443,6 +474,7 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
     __shared__ Smem s;
     Ctx c;
     c.trace_edges = nullptr;
+    c.ring_cap = 0;
     c.qn = 0;
     c.pushes = 0;
     c.edges = 0;
@@ -472,6 +504,143 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
     }
 }
 
+// ---------------------------------------------------------------- asynchronous schedule
+//
+// PPR_MODE_ASYNC: the same Alg 4 operations on every frontier vertex (eager
+// r_u read, crossing-test enqueue, fused self-update), but without rounds.
+// The frontier is one ring queue per phase: producers reserve slots with
+// atomicAdd(tail) (per warp slice / per tile flush), CTAs claim chunks with
+// atomicAdd(head) and process each chunk as a tile as soon as its slots are
+// filled, consumers free slots after reading them.  Lemma 1
+// allows any push order; within a phase residuals stay monotone, so each
+// vertex is still enqueued exactly once per crossing and is in the queue at
+// most once at a time (capacity S*n suffices; the ring has 2*S*n slots).
+// Termination: `done` counts processed entries and `tail` enqueued ones; an
+// entry's children are added to tail before the entry is added to done, so
+// reading done == tail (done first) means no entry is queued or in progress.
+
+template <bool POS>
+__device__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
+    DevCtl* ctl = a.ctl;
+    unsigned long long* head = &ctl->tilectr[0].v;
+    unsigned long long* tail = &ctl->fcount[0].v;
+    unsigned long long* done = &ctl->fcount[1].v;
+    c.Fout = a.ring;
+    c.cnt_out = tail;
+    c.ring_cap = a.ring_cap;
+    seed_phase<POS>(s, c, a);
+    block_flush(s, c);
+    grid_sync(ctl);
+    __shared__ unsigned long long s_h, s_k;
+    __shared__ int s_flag;
+    unsigned long long debt_lo = 0, debt_hi = 0;  // thread 0: claimed, not yet served
+    while (true) {
+        if (threadIdx.x == 0) {
+            unsigned long long h0 = 0, k0 = 0;
+            int flag = 0, spins = 0;
+            while (true) {
+                const unsigned long long t = *(volatile unsigned long long*)tail;
+                if (debt_lo < debt_hi) {
+                    if (t > debt_lo) {
+                        h0 = debt_lo;
+                        k0 = (t < debt_hi ? t : debt_hi) - debt_lo;
+                        debt_lo += k0;
+                        break;
+                    }
+                } else {
+                    const unsigned long long h = *(volatile unsigned long long*)head;
+                    if (t > h) {
+                        unsigned long long want = (t - h + gridDim.x - 1) / gridDim.x;
+                        want = want < 32 ? 32 : (want > PT ? PT : want);
+                        debt_lo = atomicAdd(head, want);
+                        debt_hi = debt_lo + want;
+                        continue;
+                    }
+                }
+                const unsigned long long d = *(volatile unsigned long long*)done;
+                const unsigned long long t2 = *(volatile unsigned long long*)tail;
+                if (d == t2) {
+                    flag = 1;
+                    break;
+                }
+                __nanosleep(spins < 16 ? 64 : 512);
+                spins++;
+            }
+            s_h = h0;
+            s_k = k0;
+            s_flag = flag;
+        }
+        __syncthreads();
+        if (s_flag) break;
+        const unsigned long long h = s_h;
+        const uint32_t k = (uint32_t)s_k;
+        // thread i takes slot h + i: wait for its producer, read, free the slot
+        const bool valid = threadIdx.x < k;
+        unsigned long long ent = 0;
+        if (valid) {
+            const unsigned long long pos = (h + threadIdx.x) % a.ring_cap;
+            volatile unsigned long long* slot = (volatile unsigned long long*)&a.ring[pos];
+            while ((ent = *slot) == EMPTY) __nanosleep(32);
+            *slot = EMPTY;
+        }
+        int top = 1;
+        while (top * 2 < (int)k) top <<= 1;
+        tile_body<POS, K_OPT>(s, c, a, valid, ent, 0, k, top);
+        block_flush(s, c);  // this tile's children reach `tail` ...
+        if (threadIdx.x == 0) atomicAdd(done, (unsigned long long)k);  // ... before it counts as done
+    }
+    grid_sync(ctl);
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+        *head = 0;
+        *tail = 0;
+        *done = 0;
+    }
+    grid_sync(ctl);
+}
+
+__global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid_constant__ PushArgs a) {
+    __shared__ Smem s;
+    Ctx c;
+    c.trace_edges = nullptr;
+    c.ring_cap = 0;
+    c.qn = 0;
+    c.pushes = 0;
+    c.edges = 0;
+    if (*(volatile int*)&a.ctl->st.err != KERR_OK) return;  // earlier stage failed: uniform exit
+    c.pool = *(volatile unsigned*)&a.ctl->st.active_pool ? a.g.pool[1] : a.g.pool[0];
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+        for (int i = 0; i < 3; i++) a.ctl->fcount[i].v = a.ctl->tilectr[i].v = 0;
+    }
+    grid_sync(a.ctl);
+    if (a.phases & 1) async_phase<true>(s, c, a);
+    if (a.phases & 2) async_phase<false>(s, c, a);
+    __shared__ unsigned long long s_red[2];
+    if (threadIdx.x == 0) s_red[0] = s_red[1] = 0;
+    __syncthreads();
+    if (c.pushes) atomicAdd(&s_red[0], c.pushes);
+    if (c.edges) atomicAdd(&s_red[1], c.edges);
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        if (s_red[0]) atomicAdd(&a.ctl->st.pushes, s_red[0]);
+        if (s_red[1]) atomicAdd(&a.ctl->st.pushed_edges, s_red[1]);
+    }
+}
+
+cudaError_t launch_async(const PushArgs& a, int num_sms, cudaStream_t st) {
+    static int blocks_per_sm = 0;
+    if (blocks_per_sm == 0) {
+        cudaError_t e =
+            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push_async, PT, 0);
+        if (e != cudaSuccess) return e;
+        if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
+        if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
+    }
+    dim3 grid(num_sms * blocks_per_sm), block(PT);
+    PushArgs copy = a;
+    void* args[] = {&copy};
+    return cudaLaunchCooperativeKernel((const void*)k_push_async, grid, block, args, 0, st);
+}
+
 template <int MODE>
 cudaError_t launch_mode(const PushArgs& a, int num_sms, cudaStream_t st) {
     static int blocks_per_sm = 0;
@@ -496,6 +665,7 @@ cudaError_t launch_push(int mode, const PushArgs& a, int num_sms, cudaStream_t s
         case M_EAGER: return launch_mode<M_EAGER>(a, num_sms, st);
         case M_DUP: return launch_mode<M_DUP>(a, num_sms, st);
         case M_VAN: return launch_mode<M_VAN>(a, num_sms, st);
+        case M_ASYNC: return launch_async(a, num_sms, st);
         default: return cudaErrorInvalidValue;
     }
 }

@@ -25,6 +25,8 @@ struct PushArgs {
     int phases;                // bit 0: POS, bit 1: NEG
     uint32_t max_iters;        // 0: unlimited (run to eps)
     uint32_t iter_cap;         // safety cap -> KERR_NOCONV
+    unsigned long long* ring;  // async mode: ring queue of ring_cap slots, all EMPTY between calls
+    unsigned long long ring_cap;
     unsigned long long* trace; // optional: 4 words per round {C | phase<<63, t_ns, edges, -}
     uint32_t trace_cap;        // rounds the trace buffer holds
 };

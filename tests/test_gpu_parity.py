@@ -19,7 +19,7 @@ from tests import golden_figs as G
 
 pytestmark = pytest.mark.gpu
 
-MODES = ["opt", "eager", "dupdetect", "vanilla"]
+MODES = ["opt", "eager", "dupdetect", "vanilla", "async"]
 
 
 def _fig_gpu(mode="vanilla", max_iters=0):

@@ -52,7 +52,8 @@ struct ppr_ctx {
     unsigned active = 0;     // host mirror of DevCtl::active_pool
     uint64_t pool_cap[2] = {0, 0};
     // device state
-    uint32_t* d_dout = nullptr;
+    VRec* d_rec = nullptr;       // packed layout (S == 1, pools < 2^32 entries)
+    uint32_t* d_dout = nullptr;  // structure-of-arrays layout (S > 1)
     Slab* d_slab = nullptr;
     uint32_t* d_pool[2] = {nullptr, nullptr};
     double* d_P = nullptr;
@@ -136,6 +137,7 @@ DevGraph graph_of(const ppr_ctx* h) {
     g.P = h->d_P;
     g.R = h->d_R;
     g.sources = h->d_sources;
+    g.rec = h->d_rec;
     return g;
 }
 
@@ -259,7 +261,7 @@ PushArgs push_args(ppr_ctx* h) {
     a.max_iters = h->max_iters;
     a.iter_cap = 1000000;
     if (h->d_trace) {
-        cudaMemsetAsync(h->d_trace, 0, sizeof(unsigned long long) * 4 * h->trace_cap, h->st);
+        cudaMemsetAsync(h->d_trace, 0, sizeof(unsigned long long) * (4 * h->trace_cap + 8), h->st);
         a.trace = h->d_trace;
         a.trace_cap = h->trace_cap;
     }
@@ -269,7 +271,7 @@ PushArgs push_args(ppr_ctx* h) {
 // PPR_TRACE=1: print the per-round frontier sizes, times and edges of the last push
 void dump_trace(ppr_ctx* h, const char* what) {
     if (!h->d_trace) return;
-    std::vector<unsigned long long> t(4ull * h->trace_cap);
+    std::vector<unsigned long long> t(4ull * h->trace_cap + 8);
     cudaMemcpy(t.data(), h->d_trace, sizeof(unsigned long long) * t.size(), cudaMemcpyDeviceToHost);
     fprintf(stderr, "PPR_TRACE %s:", what);
     for (uint32_t i = 0; i + 1 < h->trace_cap; i++) {
@@ -278,6 +280,11 @@ void dump_trace(ppr_ctx* h, const char* what) {
         fprintf(stderr, " [%c%llu %llu %.1fus]", (t[4 * i] >> 63) ? 'N' : 'P',
                 t[4 * i] & ~(1ull << 63), t[4 * i + 2], t1 ? (t1 - t[4 * i + 1]) / 1e3 : -1.0);
     }
+    const unsigned long long* x = &t[4ull * h->trace_cap];
+    if (x[3])
+        fprintf(stderr, "\nPPR_TRACE split per CTA (us): tiles %.1f [prologue %.1f claim %.1f] flush %.1f barrier %.1f (%llu CTAs)",
+                x[0] / 1e3 / x[3], x[4] / 1e3 / x[3], x[5] / 1e3 / x[3], x[1] / 1e3 / x[3],
+                x[2] / 1e3 / x[3], x[3]);
     fprintf(stderr, "\n");
 }
 
@@ -314,6 +321,7 @@ void record(ppr_ctx* h, int i) {
 void destroy_all(ppr_ctx* h) {
     if (h->st) cudaStreamSynchronize(h->st);
     free_batch(h);
+    dfree(h, h->d_rec, h->n);
     dfree(h, h->d_dout, h->n);
     dfree(h, h->d_slab, h->n);
     dfree(h, h->d_pool[0], h->pool_cap[0]);
@@ -336,7 +344,7 @@ void destroy_all(ppr_ctx* h) {
     h->h_ctl = nullptr;
     for (auto& e : h->ev)
         if (e) cudaEventDestroy(e), e = nullptr;
-    dfree(h, h->d_trace, 4ull * h->trace_cap);
+    dfree(h, h->d_trace, 4ull * h->trace_cap + 8);
     dfree(h, h->d_ring, h->ring_cap);
     if (h->own_stream && h->st) cudaStreamDestroy(h->st);
     h->st = nullptr;
@@ -443,13 +451,23 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     h->npasses = key_shifts(ceil_log2(h->n), h->shifts);
     if (getenv("PPR_TRACE") && atoi(getenv("PPR_TRACE")) > 0) {
         h->trace_cap = 4096;
-        dalloc(h, &h->d_trace, 4ull * h->trace_cap);
+        dalloc(h, &h->d_trace, 4ull * h->trace_cap + 8);
     }
 
     const uint64_t Sn = (uint64_t)h->S * h->n;
     const uint64_t arcs_in = g->undirected ? 2 * g->m : g->m;
-    bool ok = dalloc(h, &h->d_dout, h->n) == cudaSuccess && dalloc(h, &h->d_slab, h->n) == cudaSuccess &&
-              dalloc(h, &h->d_P, Sn) == cudaSuccess && dalloc(h, &h->d_R, Sn) == cudaSuccess &&
+    // layout: one 32-byte record per vertex for single-source handles whose
+    // pools fit 32-bit offsets; arrays (R, P as [S][n]) otherwise
+    const double pool_bound = (1.0 + h->slack) * (double)arcs_in * 1.25 + 8.0 * h->n + 4096;
+    // Default: arrays (R + d_out = 12 B/vertex stay L2-resident, see ppr_internal.cuh);
+    // PPR_LAYOUT=packed selects the 32-byte records for experiments.
+    const char* lay = getenv("PPR_LAYOUT");
+    const bool packed = lay && !strcmp(lay, "packed") && h->S == 1 && pool_bound < 4.0e9;
+    bool ok = packed ? dalloc(h, &h->d_rec, h->n) == cudaSuccess
+                     : (dalloc(h, &h->d_dout, h->n) == cudaSuccess &&
+                        dalloc(h, &h->d_slab, h->n) == cudaSuccess &&
+                        dalloc(h, &h->d_P, Sn) == cudaSuccess && dalloc(h, &h->d_R, Sn) == cudaSuccess);
+    ok = ok &&
               dalloc(h, &h->d_sources, h->S) == cudaSuccess &&
               dalloc(h, &h->d_F[0], Sn) == cudaSuccess && dalloc(h, &h->d_F[1], Sn) == cudaSuccess &&
               dalloc(h, &h->d_W, Sn) == cudaSuccess &&
@@ -474,10 +492,14 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     cudaStream_t st = h->st;
     record(h, 0);
     cudaMemsetAsync(h->d_ctl, 0, sizeof(DevCtl), st);
-    cudaMemsetAsync(h->d_dout, 0, sizeof(uint32_t) * h->n, st);
-    cudaMemsetAsync(h->d_slab, 0, sizeof(Slab) * h->n, st);
-    cudaMemsetAsync(h->d_P, 0, sizeof(double) * Sn, st);
-    cudaMemsetAsync(h->d_R, 0, sizeof(double) * Sn, st);
+    if (packed) {
+        cudaMemsetAsync(h->d_rec, 0, sizeof(VRec) * h->n, st);
+    } else {
+        cudaMemsetAsync(h->d_dout, 0, sizeof(uint32_t) * h->n, st);
+        cudaMemsetAsync(h->d_slab, 0, sizeof(Slab) * h->n, st);
+        cudaMemsetAsync(h->d_P, 0, sizeof(double) * Sn, st);
+        cudaMemsetAsync(h->d_R, 0, sizeof(double) * Sn, st);
+    }
     cudaMemsetAsync(h->d_bitmap, 0, sizeof(uint32_t) * ((Sn + 31) / 32), st);
     cudaMemsetAsync(h->vb.vseg, 0xFF, sizeof(uint32_t) * h->n, st);
     cudaMemcpyAsync(h->d_sources, sources, sizeof(uint32_t) * h->S, cudaMemcpyHostToDevice, st);
@@ -556,10 +578,16 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         return rs;
     }
     if (h->undirected) {  // exact arc count (self-loops once)
-        std::vector<Slab> sl(h->n);
-        cudaMemcpy(sl.data(), h->d_slab, sizeof(Slab) * h->n, cudaMemcpyDeviceToHost);
+        uint32_t* lens = nullptr;
         uint64_t mm = 0;
-        for (auto& x : sl) mm += x.len;
+        if (dalloc(h, &lens, h->n) == cudaSuccess) {
+            launch_len_to_u32(graph_of(h), lens, h->st, &launches);
+            std::vector<uint32_t> hl(h->n);
+            cudaMemcpyAsync(hl.data(), lens, sizeof(uint32_t) * h->n, cudaMemcpyDeviceToHost, h->st);
+            cudaStreamSynchronize(h->st);
+            for (uint32_t x : hl) mm += x;
+            dfree(h, lens, h->n);
+        }
         h->m = mm;
     }
     fill_stats(h, stats, launches, h->timing);
@@ -702,8 +730,12 @@ ppr_status ppr_reset(ppr_ctx* h) {
     if (h->poisoned) return PPR_EPOISONED;
     uint32_t launches = 0;
     const uint64_t Sn = (uint64_t)h->S * h->n;
-    cudaMemsetAsync(h->d_P, 0, sizeof(double) * Sn, h->st);
-    cudaMemsetAsync(h->d_R, 0, sizeof(double) * Sn, h->st);
+    if (h->d_rec) {
+        launch_gather_rec(graph_of(h), nullptr, nullptr, nullptr, 1, h->st, &launches);
+    } else {
+        cudaMemsetAsync(h->d_P, 0, sizeof(double) * Sn, h->st);
+        cudaMemsetAsync(h->d_R, 0, sizeof(double) * Sn, h->st);
+    }
     launch_init_state(graph_of(h), h->st, &launches);
     cudaError_t e = cudaStreamSynchronize(h->st);
     if (e == cudaSuccess) e = cudaGetLastError();
@@ -719,6 +751,22 @@ ppr_status ppr_query(ppr_ctx* h, uint32_t source_idx, double* P_out, double* R_o
     const cudaMemcpyKind k = mem == PPR_MEM_HOST ? cudaMemcpyDeviceToHost : cudaMemcpyDeviceToDevice;
     const size_t off = (size_t)source_idx * h->n;
     cudaError_t e = cudaSuccess;
+    if (h->d_rec) {  // gather out of the vertex records (through a device buffer for host output)
+        double* tmp = nullptr;
+        const bool host = mem == PPR_MEM_HOST;
+        if (host && dalloc(h, &tmp, 2ull * h->n) != cudaSuccess) return PPR_ENOMEM;
+        uint32_t launches = 0;
+        double* dP = host ? (P_out ? tmp : nullptr) : P_out;
+        double* dR = host ? (R_out ? tmp + h->n : nullptr) : R_out;
+        launch_gather_rec(graph_of(h), dP, dR, nullptr, 0, h->st, &launches);
+        if (host && P_out) e = cudaMemcpyAsync(P_out, tmp, sizeof(double) * h->n, k, h->st);
+        if (host && e == cudaSuccess && R_out)
+            e = cudaMemcpyAsync(R_out, tmp + h->n, sizeof(double) * h->n, k, h->st);
+        if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
+        dfree(h, tmp, 2ull * h->n);
+        if (e != cudaSuccess) return cuda_fail(h, e, "ppr_query");
+        return PPR_OK;
+    }
     if (P_out) e = cudaMemcpyAsync(P_out, h->d_P + off, sizeof(double) * h->n, k, h->st);
     if (e == cudaSuccess && R_out) e = cudaMemcpyAsync(R_out, h->d_R + off, sizeof(double) * h->n, k, h->st);
     if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
@@ -729,7 +777,19 @@ ppr_status ppr_query(ppr_ctx* h, uint32_t source_idx, double* P_out, double* R_o
 ppr_status ppr_export_dout(ppr_ctx* h, uint32_t* dout_out) {
     if (!h || !dout_out) return PPR_EINVAL;
     if (h->poisoned) return PPR_EPOISONED;
-    cudaError_t e = cudaMemcpyAsync(dout_out, h->d_dout, sizeof(uint32_t) * h->n,
+    cudaError_t e = cudaSuccess;
+    if (h->d_rec) {
+        uint32_t* tmp = nullptr;
+        uint32_t launches = 0;
+        if (dalloc(h, &tmp, h->n) != cudaSuccess) return PPR_ENOMEM;
+        launch_gather_rec(graph_of(h), nullptr, nullptr, tmp, 0, h->st, &launches);
+        e = cudaMemcpyAsync(dout_out, tmp, sizeof(uint32_t) * h->n, cudaMemcpyDeviceToHost, h->st);
+        if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
+        dfree(h, tmp, h->n);
+        if (e != cudaSuccess) return cuda_fail(h, e, "ppr_export_dout");
+        return PPR_OK;
+    }
+    e = cudaMemcpyAsync(dout_out, h->d_dout, sizeof(uint32_t) * h->n,
                                     cudaMemcpyDeviceToHost, h->st);
     if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, "ppr_export_dout");

@@ -22,6 +22,18 @@ struct __align__(16) Slab {
     uint32_t cap;            // reserved entries
 };
 
+// Packed layout (single-source handles): every per-vertex field the hot path
+// touches lives in one 32-byte record = one DRAM/L2 sector, so a pushed
+// vertex (R, P, slab) and an edge target (R, d_out) each cost one sector.
+struct __align__(32) VRec {
+    double r;       // R_s(v)
+    double p;       // P_s(v)
+    uint32_t off;   // first pool index of N_in(v)
+    uint32_t len;   // |N_in(v)|
+    uint32_t dout;  // d_out(v)
+    uint32_t cap;   // reserved slab entries
+};
+
 // error codes written by kernels into DevCtl::err (mirror ppr_status)
 enum : int { KERR_OK = 0, KERR_RANGE = -2, KERR_NOENT = -3, KERR_NOCONV = -7, KERR_OVERFLOW = -8 };
 
@@ -74,7 +86,55 @@ struct DevGraph {
     double* P;
     double* R;
     const uint32_t* sources;  // [S]
+    VRec* rec;                // packed layout (S == 1): replaces dout, slab, R, P
 };
+
+// ------------------------------------------------------------------ layout accessors
+// PK = packed (VRec) layout; otherwise structure of arrays with R, P as [S][n].
+
+template <bool PK>
+__device__ __forceinline__ double* Rp(const DevGraph& g, uint32_t sidx, uint32_t v) {
+    if (PK) return &g.rec[v].r;
+    return g.R + (size_t)sidx * g.n + v;
+}
+template <bool PK>
+__device__ __forceinline__ double* Pp(const DevGraph& g, uint32_t sidx, uint32_t v) {
+    if (PK) return &g.rec[v].p;
+    return g.P + (size_t)sidx * g.n + v;
+}
+template <bool PK>
+__device__ __forceinline__ uint32_t* doutp(const DevGraph& g, uint32_t v) {
+    if (PK) return &g.rec[v].dout;
+    return &g.dout[v];
+}
+template <bool PK>
+__device__ __forceinline__ uint32_t* lenp(const DevGraph& g, uint32_t v) {
+    if (PK) return &g.rec[v].len;
+    return &g.slab[v].len;
+}
+template <bool PK>
+__device__ __forceinline__ Slab get_slab(const DevGraph& g, uint64_t v) {
+    Slab s;
+    if (PK) {
+        const uint4 q = __ldcg(reinterpret_cast<const uint4*>(&g.rec[v].off));
+        s.off = q.x;
+        s.len = q.y;
+        s.cap = q.w;
+    } else {
+        s = g.slab[v];
+    }
+    return s;
+}
+template <bool PK>
+__device__ __forceinline__ void put_slab(const DevGraph& g, uint64_t v, const Slab& s) {
+    if (PK) {
+        g.rec[v].off = (uint32_t)s.off;
+        g.rec[v].len = s.len;
+        g.rec[v].cap = s.cap;
+    } else {
+        g.slab[v] = s;
+    }
+}
 
 // ------------------------------------------------------------------ helpers
 
@@ -120,6 +180,44 @@ __device__ __forceinline__ void grid_sync(DevCtl* ctl) {
 }
 
 __device__ __forceinline__ unsigned lane_id() { return threadIdx.x & 31u; }
+
+// ------------------------------------------------------------------ L2 cache policies
+// The push is bound by random fp64 atomics: ~120 G/s when the residual array
+// is L2-resident vs ~43 G/s once it spills to DRAM (tools/atomic_bench.cu on
+// B200).  R and d_out (the per-edge random targets) are therefore accessed
+// with an evict_last policy and the streamed data (slab pool, descriptors,
+// P, frontiers) with evict_first.
+__device__ __forceinline__ unsigned long long l2_keep() {
+    unsigned long long p;
+    asm("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+__device__ __forceinline__ unsigned long long l2_stream() {
+    unsigned long long p;
+    asm("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+__device__ __forceinline__ double atom_add_pol(double* a, double v, unsigned long long pol) {
+    double r;
+    asm volatile("atom.global.add.L2::cache_hint.f64 %0, [%1], %2, %3;"
+                 : "=d"(r) : "l"(a), "d"(v), "l"(pol) : "memory");
+    return r;
+}
+__device__ __forceinline__ void red_add_pol(double* a, double v, unsigned long long pol) {
+    asm volatile("red.global.add.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(a), "d"(v), "l"(pol)
+                 : "memory");
+}
+__device__ __forceinline__ uint32_t ld_u32_pol(const uint32_t* a, unsigned long long pol) {
+    uint32_t r;
+    asm volatile("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
+    return r;
+}
+__device__ __forceinline__ ulonglong2 ld_u64x2_pol(const void* a, unsigned long long pol) {
+    ulonglong2 r;
+    asm volatile("ld.global.nc.L2::cache_hint.v2.u64 {%0, %1}, [%2], %3;"
+                 : "=l"(r.x), "=l"(r.y) : "l"(a), "l"(pol));
+    return r;
+}
 
 // pushCond of Alg 3 lines 8-10: POS r > eps, NEG r < -eps
 template <bool POS>

@@ -79,6 +79,8 @@ struct Ctx {
     uint32_t qn;                      // warp-uniform fill of this warp's slice
     unsigned long long pushes;        // per-thread counters
     unsigned long long edges;
+    unsigned long long t_work, t_flush, t_bar;  // trace mode: ns per CTA in tiles / flush / barrier
+    unsigned long long t_pro, t_claim, t_mark, t_mark2;  // tile prologue, claims
 };
 
 __device__ __forceinline__ unsigned lane() { return threadIdx.x & 31u; }
@@ -163,7 +165,7 @@ __device__ __forceinline__ int owner_of(const uint32_t* scan, uint32_t e, int to
 
 // ---------------------------------------------------------------- CTA tile
 
-template <bool POS, int KIND>
+template <bool POS, int KIND, bool PK>
 __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
                                           unsigned long long ent, uint64_t idx, uint32_t T,
                                           int top);
@@ -171,18 +173,18 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
 // Processes the T entries Fin[base_idx .. base_idx+T) (thread i = entry i):
 // neighbour propagation of every pushed entry and, for K_OPT, the fused
 // self-update.  Must be called by all threads of the CTA.
-template <bool POS, int KIND>
+template <bool POS, int KIND, bool PK>
 __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
                                          const unsigned long long* Fin, uint64_t C,
                                          uint64_t base_idx, uint32_t T, int top) {
     const uint64_t idx = base_idx + threadIdx.x;
     const bool valid = threadIdx.x < T && idx < C;
     const unsigned long long ent = valid ? __ldcg(&Fin[idx]) : 0ull;
-    tile_body<POS, KIND>(s, c, a, valid, ent, idx, T, top);
+    tile_body<POS, KIND, PK>(s, c, a, valid, ent, idx, T, top);
 }
 
 // The tile's work once thread i holds entry i (valid, ent; idx indexes W).
-template <bool POS, int KIND>
+template <bool POS, int KIND, bool PK>
 __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
                                           unsigned long long ent, uint64_t idx, uint32_t T,
                                           int top) {
@@ -190,7 +192,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     const double eps = a.g.eps, alpha = a.g.alpha;
     const uint32_t n = a.g.n;
     const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
-    double* ru = a.g.R + (size_t)sidx * n + u;
+    double* ru = Rp<PK>(a.g, sidx, u);
     double r = 0.0;
     bool push = false;
     if (KIND == K_OPT || KIND == K_EAGER) {
@@ -213,14 +215,20 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     double self_old = 0.0;
     if (KIND == K_OPT && push) {
         self_old = atomicAdd(ru, -r);
-        atomicAdd(a.g.P + (size_t)sidx * n + u, __dmul_rn(alpha, r));
+        red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
     }
     uint32_t len = 0;
     unsigned long long off = 0;
     if (push) {
-        const ulonglong2 sl = __ldg(reinterpret_cast<const ulonglong2*>(&a.g.slab[u]));
-        off = sl.x;               // Slab::off
-        len = (uint32_t)sl.y;     // Slab::len (low word of {len, cap})
+        if (PK) {  // {off, len} of the vertex record (same sector as R(u), P(u))
+            const uint2 q = __ldcg(reinterpret_cast<const uint2*>(&a.g.rec[u].off));
+            off = q.x;
+            len = q.y;
+        } else {
+            const ulonglong2 sl = ld_u64x2_pol(&a.g.slab[u], l2_stream());
+            off = sl.x;               // Slab::off
+            len = (uint32_t)sl.y;     // Slab::len (low word of {len, cap})
+        }
     }
     uint32_t E;
     const uint32_t ex = block_exclusive_scan_u32<PT>(len, s.warp_tmp, &E);
@@ -230,10 +238,12 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     s.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
     s.sid[threadIdx.x] = sidx;
     __syncthreads();
+    if (a.trace && threadIdx.x == 0) c.t_pro += global_ns() - c.t_mark;
     if (threadIdx.x == 0) {
         c.edges += E;
         if (c.trace_edges && E) atomicAdd(c.trace_edges, (unsigned long long)E);
     }
+    const unsigned long long pol_keep = l2_keep(), pol_stream = l2_stream();
     // 32-edge chunks dealt round-robin to the warps (chunk w + NW*i), U per step
     for (uint32_t cb = w; cb * 32 < E; cb += NW * U) {
         ensure_room(s, c, 32 * U);
@@ -246,12 +256,13 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             v[k] = 0;
             if (e < E) {
                 j[k] = owner_of(s.scan, e, top);
-                v[k] = __ldg(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])]);
+                v[k] = ld_u32_pol(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
             }
         }
         uint32_t d[U];
 #pragma unroll
-        for (int k = 0; k < U; k++) d[k] = j[k] >= 0 ? __ldg(&a.g.dout[v[k]]) : 1u;
+        for (int k = 0; k < U; k++)
+            d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_pol(&a.g.dout[v[k]], pol_keep));
 #pragma unroll
         for (int k = 0; k < U; k++) {
             bool enq = false;
@@ -259,7 +270,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             if (j[k] >= 0) {
                 const uint32_t sj = s.sid[j[k]];
                 const double incr = __ddiv_rn(s.w[j[k]], (double)d[k]);
-                const double pre = atomicAdd(a.g.R + (size_t)sj * n + v[k], incr);
+                const double pre = atom_add_pol(Rp<PK>(a.g, sj, v[k]), incr, pol_keep);
                 const double cur = __dadd_rn(pre, incr);  // == the stored value (no FMA)
                 ev = ((unsigned long long)sj << 32) | v[k];
                 if (KIND == K_OPT || KIND == K_DUP)
@@ -284,7 +295,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
 
 // Every CTA takes tiles of T entries: its first tile statically, the rest by
 // one atomic claim each, until C is covered.
-template <bool POS, int KIND>
+template <bool POS, int KIND, bool PK>
 __device__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a, const unsigned long long* Fin,
                               uint64_t C, unsigned long long* tc) {
     uint64_t per = (C + gridDim.x - 1) / gridDim.x;
@@ -296,18 +307,22 @@ __device__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a, const unsigned
     const uint64_t ntiles = (C + T - 1) / T;
     uint64_t t = blockIdx.x;
     while (t < ntiles) {
-        cta_tile<POS, KIND>(s, c, a, Fin, C, t * T, T, top);
+        if (a.trace && threadIdx.x == 0) c.t_mark = global_ns();
+        cta_tile<POS, KIND, PK>(s, c, a, Fin, C, t * T, T, top);
+        if (a.trace && threadIdx.x == 0) c.t_mark2 = global_ns();
         if (ntiles <= gridDim.x) break;  // every tile was assigned statically
         if (threadIdx.x == 0) s.next = atomicAdd(tc, 1ull) + gridDim.x;
         __syncthreads();
         t = s.next;
         __syncthreads();
+        if (a.trace && threadIdx.x == 0) c.t_claim += global_ns() - c.t_mark2;
     }
 }
 
 // ---------------------------------------------------------------- Alg 3 / Eager sessions
 
 // self-update session of Alg 3 (lines 13-16): w = R(u), P(u) += a w, R(u) = 0
+template <bool PK>
 __device__ void session_snapshot(Ctx& c, const PushArgs& a, const unsigned long long* Fin,
                                  uint64_t C, bool bitmap) {
     const double alpha = a.g.alpha;
@@ -315,9 +330,11 @@ __device__ void session_snapshot(Ctx& c, const PushArgs& a, const unsigned long 
          idx += (uint64_t)gridDim.x * PT) {
         const unsigned long long ent = __ldcg(&Fin[idx]);
         const size_t i = (size_t)(ent >> 32) * a.g.n + (uint32_t)ent;
-        const double w = __ldcg(&a.g.R[i]);
-        __stcg(&a.g.P[i], __dadd_rn(__ldcg(&a.g.P[i]), __dmul_rn(alpha, w)));
-        __stcg(&a.g.R[i], 0.0);
+        double* rp = Rp<PK>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent);
+        double* pp = Pp<PK>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent);
+        const double w = __ldcg(rp);
+        __stcg(pp, __dadd_rn(__ldcg(pp), __dmul_rn(alpha, w)));
+        __stcg(rp, 0.0);
         __stcg(&a.W[idx], w);
         if (bitmap) clear_bit(a.bitmap, i);
         c.pushes++;
@@ -325,7 +342,7 @@ __device__ void session_snapshot(Ctx& c, const PushArgs& a, const unsigned long 
 }
 
 // Eager: self-update with the r_u recorded during propagation (Alg 4 lines 19-23)
-template <bool POS>
+template <bool POS, bool PK>
 __device__ void session_eager_self(Smem& s, Ctx& c, const PushArgs& a,
                                    const unsigned long long* Fin, uint64_t C) {
     const double eps = a.g.eps, alpha = a.g.alpha;
@@ -339,9 +356,9 @@ __device__ void session_eager_self(Smem& s, Ctx& c, const PushArgs& a,
             const double r = __ldcg(&a.W[idx]);
             if (r != 0.0) {
                 const size_t i = (size_t)(ent >> 32) * a.g.n + (uint32_t)ent;
-                const double old = atomicAdd(&a.g.R[i], -r);
+                const double old = atomicAdd(Rp<PK>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent), -r);
                 const double cur = __dadd_rn(old, -r);
-                __stcg(&a.g.P[i], __dadd_rn(__ldcg(&a.g.P[i]), __dmul_rn(alpha, r)));
+                atomicAdd(Pp<PK>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent), __dmul_rn(alpha, r));
                 c.pushes++;
                 enq = push_cond<POS>(cur, eps) && test_and_set(a.bitmap, i);
             }
@@ -362,7 +379,7 @@ __device__ void clear_frontier_bits(Ctx& c, const PushArgs& a, const unsigned lo
 
 // ---------------------------------------------------------------- seeding
 
-template <bool POS>
+template <bool POS, bool PK>
 __device__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
     const double eps = a.g.eps;
     const uint64_t stride = (uint64_t)gridDim.x * PT;
@@ -392,7 +409,7 @@ __device__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
                 v = (uint32_t)ent;
             }
             ent = ((unsigned long long)sidx << 32) | v;
-            enq = push_cond<POS>(__ldcg(&a.g.R[(size_t)sidx * a.g.n + v]), eps);
+            enq = push_cond<POS>(__ldcg(Rp<PK>(a.g, sidx, v)), eps);
         }
         ensure_room(s, c, 32);
         warp_enqueue(s, c, enq, ent);
@@ -401,14 +418,14 @@ __device__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
 
 // ---------------------------------------------------------------- phase driver
 
-template <int MODE, bool POS>
+template <int MODE, bool POS, bool PK>
 __device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
     DevCtl* ctl = a.ctl;
     const int ph = POS ? 0 : 1;
     // seed into F[it%2] / fcount[it%3]; both that and the next counter are 0 here
     c.Fout = a.F[it & 1];
     c.cnt_out = &ctl->fcount[it % 3].v;
-    seed_phase<POS>(s, c, a);
+    seed_phase<POS, PK>(s, c, a);
     block_flush(s, c);
     grid_sync(ctl);
     uint32_t pit = 0;
@@ -437,24 +454,33 @@ __device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
         c.Fout = a.F[(it + 1) & 1];
         c.cnt_out = &ctl->fcount[(it + 1) % 3].v;
         unsigned long long* tc = &ctl->tilectr[it % 3].v;
+        const unsigned long long t0 = a.trace ? global_ns() : 0;
         if (MODE == M_OPT) {
-            propagate_all<POS, K_OPT>(s, c, a, Fin, C, tc);
+            propagate_all<POS, K_OPT, PK>(s, c, a, Fin, C, tc);
         } else if (MODE == M_VAN || MODE == M_DUP) {
-            session_snapshot(c, a, Fin, C, MODE == M_VAN);
+            session_snapshot<PK>(c, a, Fin, C, MODE == M_VAN);
             grid_sync(ctl);
             if (MODE == M_VAN)
-                propagate_all<POS, K_VAN>(s, c, a, Fin, C, tc);
+                propagate_all<POS, K_VAN, PK>(s, c, a, Fin, C, tc);
             else
-                propagate_all<POS, K_DUP>(s, c, a, Fin, C, tc);
+                propagate_all<POS, K_DUP, PK>(s, c, a, Fin, C, tc);
         } else {  // M_EAGER
             clear_frontier_bits(c, a, Fin, C);
             grid_sync(ctl);
-            propagate_all<POS, K_EAGER>(s, c, a, Fin, C, tc);
+            propagate_all<POS, K_EAGER, PK>(s, c, a, Fin, C, tc);
             grid_sync(ctl);
-            session_eager_self<POS>(s, c, a, Fin, C);
+            session_eager_self<POS, PK>(s, c, a, Fin, C);
         }
+        const unsigned long long t1 = a.trace ? global_ns() : 0;
         block_flush(s, c);
+        const unsigned long long t2 = a.trace ? global_ns() : 0;
         grid_sync(ctl);
+        if (a.trace) {
+            const unsigned long long t3 = global_ns();
+            c.t_work += t1 - t0;
+            c.t_flush += t2 - t1;
+            c.t_bar += t3 - t2;
+        }
         it++;
         pit++;
     }
@@ -469,7 +495,7 @@ __device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
     grid_sync(ctl);
 }
 
-template <int MODE>
+template <int MODE, bool PK>
 __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_constant__ PushArgs a) {
     __shared__ Smem s;
     Ctx c;
@@ -478,6 +504,8 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
     c.qn = 0;
     c.pushes = 0;
     c.edges = 0;
+    c.t_work = c.t_flush = c.t_bar = 0;
+    c.t_pro = c.t_claim = c.t_mark = c.t_mark2 = 0;
     if (*(volatile int*)&a.ctl->st.err != KERR_OK) return;  // earlier stage failed: uniform exit
     c.pool = *(volatile unsigned*)&a.ctl->st.active_pool ? a.g.pool[1] : a.g.pool[0];
     if (blockIdx.x == 0 && threadIdx.x == 0) {
@@ -485,11 +513,19 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
     }
     grid_sync(a.ctl);
     unsigned it = 0;
-    if (a.phases & 1) run_phase<MODE, true>(s, c, a, it);
-    if (a.phases & 2) run_phase<MODE, false>(s, c, a, it);
+    if (a.phases & 1) run_phase<MODE, true, PK>(s, c, a, it);
+    if (a.phases & 2) run_phase<MODE, false, PK>(s, c, a, it);
     if (a.trace && blockIdx.x == 0 && threadIdx.x == 0 && it < a.trace_cap) {
         a.trace[4ull * it] = ~0ull;  // end marker
         a.trace[4ull * it + 1] = global_ns();
+    }
+    if (a.trace && threadIdx.x == 0) {  // per-CTA time split, summed over CTAs
+        atomicAdd(&a.trace[4ull * a.trace_cap + 0], c.t_work);
+        atomicAdd(&a.trace[4ull * a.trace_cap + 1], c.t_flush);
+        atomicAdd(&a.trace[4ull * a.trace_cap + 2], c.t_bar);
+        atomicAdd(&a.trace[4ull * a.trace_cap + 3], 1ull);
+        atomicAdd(&a.trace[4ull * a.trace_cap + 4], c.t_pro);
+        atomicAdd(&a.trace[4ull * a.trace_cap + 5], c.t_claim);
     }
     // statistics
     __shared__ unsigned long long s_red[2];
@@ -519,7 +555,7 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
 // entry's children are added to tail before the entry is added to done, so
 // reading done == tail (done first) means no entry is queued or in progress.
 
-template <bool POS>
+template <bool POS, bool PK>
 __device__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
     DevCtl* ctl = a.ctl;
     unsigned long long* head = &ctl->tilectr[0].v;
@@ -528,7 +564,7 @@ __device__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
     c.Fout = a.ring;
     c.cnt_out = tail;
     c.ring_cap = a.ring_cap;
-    seed_phase<POS>(s, c, a);
+    seed_phase<POS, PK>(s, c, a);
     block_flush(s, c);
     grid_sync(ctl);
     __shared__ unsigned long long s_h, s_k;
@@ -585,7 +621,7 @@ __device__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
         }
         int top = 1;
         while (top * 2 < (int)k) top <<= 1;
-        tile_body<POS, K_OPT>(s, c, a, valid, ent, 0, k, top);
+        tile_body<POS, K_OPT, PK>(s, c, a, valid, ent, 0, k, top);
         block_flush(s, c);  // this tile's children reach `tail` ...
         if (threadIdx.x == 0) atomicAdd(done, (unsigned long long)k);  // ... before it counts as done
     }
@@ -598,6 +634,7 @@ __device__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
     grid_sync(ctl);
 }
 
+template <bool PK>
 __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid_constant__ PushArgs a) {
     __shared__ Smem s;
     Ctx c;
@@ -606,14 +643,16 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid
     c.qn = 0;
     c.pushes = 0;
     c.edges = 0;
+    c.t_work = c.t_flush = c.t_bar = 0;
+    c.t_pro = c.t_claim = c.t_mark = c.t_mark2 = 0;
     if (*(volatile int*)&a.ctl->st.err != KERR_OK) return;  // earlier stage failed: uniform exit
     c.pool = *(volatile unsigned*)&a.ctl->st.active_pool ? a.g.pool[1] : a.g.pool[0];
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         for (int i = 0; i < 3; i++) a.ctl->fcount[i].v = a.ctl->tilectr[i].v = 0;
     }
     grid_sync(a.ctl);
-    if (a.phases & 1) async_phase<true>(s, c, a);
-    if (a.phases & 2) async_phase<false>(s, c, a);
+    if (a.phases & 1) async_phase<true, PK>(s, c, a);
+    if (a.phases & 2) async_phase<false, PK>(s, c, a);
     __shared__ unsigned long long s_red[2];
     if (threadIdx.x == 0) s_red[0] = s_red[1] = 0;
     __syncthreads();
@@ -626,11 +665,12 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid
     }
 }
 
+template <bool PK>
 cudaError_t launch_async(const PushArgs& a, int num_sms, cudaStream_t st) {
     static int blocks_per_sm = 0;
     if (blocks_per_sm == 0) {
         cudaError_t e =
-            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push_async, PT, 0);
+            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push_async<PK>, PT, 0);
         if (e != cudaSuccess) return e;
         if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
         if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
@@ -638,15 +678,15 @@ cudaError_t launch_async(const PushArgs& a, int num_sms, cudaStream_t st) {
     dim3 grid(num_sms * blocks_per_sm), block(PT);
     PushArgs copy = a;
     void* args[] = {&copy};
-    return cudaLaunchCooperativeKernel((const void*)k_push_async, grid, block, args, 0, st);
+    return cudaLaunchCooperativeKernel((const void*)k_push_async<PK>, grid, block, args, 0, st);
 }
 
-template <int MODE>
+template <int MODE, bool PK>
 cudaError_t launch_mode(const PushArgs& a, int num_sms, cudaStream_t st) {
     static int blocks_per_sm = 0;
     if (blocks_per_sm == 0) {
         cudaError_t e =
-            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push<MODE>, PT, 0);
+            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push<MODE, PK>, PT, 0);
         if (e != cudaSuccess) return e;
         if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
         if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
@@ -654,20 +694,26 @@ cudaError_t launch_mode(const PushArgs& a, int num_sms, cudaStream_t st) {
     dim3 grid(num_sms * blocks_per_sm), block(PT);
     PushArgs copy = a;
     void* args[] = {&copy};
-    return cudaLaunchCooperativeKernel((const void*)k_push<MODE>, grid, block, args, 0, st);
+    return cudaLaunchCooperativeKernel((const void*)k_push<MODE, PK>, grid, block, args, 0, st);
+}
+
+template <bool PK>
+cudaError_t launch_layout(int mode, const PushArgs& a, int num_sms, cudaStream_t st) {
+    switch (mode) {
+        case M_OPT: return launch_mode<M_OPT, PK>(a, num_sms, st);
+        case M_EAGER: return launch_mode<M_EAGER, PK>(a, num_sms, st);
+        case M_DUP: return launch_mode<M_DUP, PK>(a, num_sms, st);
+        case M_VAN: return launch_mode<M_VAN, PK>(a, num_sms, st);
+        case M_ASYNC: return launch_async<PK>(a, num_sms, st);
+        default: return cudaErrorInvalidValue;
+    }
 }
 
 }  // namespace
 
 cudaError_t launch_push(int mode, const PushArgs& a, int num_sms, cudaStream_t st) {
-    switch (mode) {
-        case M_OPT: return launch_mode<M_OPT>(a, num_sms, st);
-        case M_EAGER: return launch_mode<M_EAGER>(a, num_sms, st);
-        case M_DUP: return launch_mode<M_DUP>(a, num_sms, st);
-        case M_VAN: return launch_mode<M_VAN>(a, num_sms, st);
-        case M_ASYNC: return launch_async(a, num_sms, st);
-        default: return cudaErrorInvalidValue;
-    }
+    return a.g.rec ? launch_layout<true>(mode, a, num_sms, st)
+                   : launch_layout<false>(mode, a, num_sms, st);
 }
 
 }  // namespace ppr

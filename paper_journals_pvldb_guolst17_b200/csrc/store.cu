@@ -160,6 +160,7 @@ __global__ void k_heads(const uint64_t* __restrict__ keys, const uint32_t* __res
 
 // ---------------------------------------------------------------- a1 store
 
+template <bool PK>
 __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, uint64_t N,
                                  BatchBufs b, uint32_t* __restrict__ vseg, DevCtl* ctl,
                                  int force_rebuild) {
@@ -182,7 +183,7 @@ __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, ui
         }
         I = warp_sum_u32(I);
         Dn = warp_sum_u32(Dn);
-        const Slab sl = g.slab[v];
+        const Slab sl = get_slab<PK>(g, v);
         uint32_t found = 0;
         if (Dn > 0) {
             for (uint32_t p0 = 0; p0 < sl.len && found < Dn; p0 += 32) {
@@ -215,6 +216,7 @@ __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, ui
     }
 }
 
+template <bool PK>
 __global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, BatchBufs b,
                               DevCtl* ctl) {
     if (*(volatile int*)&ctl->st.err != KERR_OK || *(volatile int*)&ctl->st.rebuild) return;
@@ -228,7 +230,7 @@ __global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, Batch
         const uint32_t v = (uint32_t)(kv[i0] >> 32);
         const uint64_t i1 = b.seg_end[i0];
         const uint32_t D = b.seg_D[i0], I = b.seg_I[i0];
-        const Slab sl = g.slab[v];
+        const Slab sl = get_slab<PK>(g, v);
         const uint32_t keep = sl.len - D;
         const uint32_t* dp = b.delpos + i0;
         // fill the holes (deleted positions < keep) with the surviving tail entries
@@ -261,7 +263,7 @@ __global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, Batch
             for (uint32_t k = 0; k < c; k++) pool[sl.off + pos + ex + k] = x;
             pos += tot;
         }
-        if (lane == 0) g.slab[v].len = keep + I;
+        if (lane == 0) *lenp<PK>(g, v) = keep + I;
     }
 }
 
@@ -276,9 +278,10 @@ __global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, Batch
 constexpr int RB_THREADS = 256;
 
 // new length of v after this batch (the batch's segment for v, if any)
+template <bool PK>
 __device__ __forceinline__ uint32_t merged_len(const DevGraph& g, const BatchBufs& b,
                                                const VertexBufs& vb, uint64_t v) {
-    uint32_t len = g.slab[v].len;
+    uint32_t len = *lenp<PK>(g, (uint32_t)v);
     const uint32_t sg = vb.vseg[v];
     if (sg != NONE) len = len - b.seg_D[sg] + b.seg_I[sg];
     return len;
@@ -326,6 +329,7 @@ __device__ uint32_t copy_merged_warp(const uint32_t* src, uint32_t* dst, const S
     return pos;
 }
 
+template <bool PK>
 __global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64_t* __restrict__ kv,
                                                         BatchBufs b, VertexBufs vb, double slack,
                                                         uint32_t min_cap, uint64_t alt_cap,
@@ -344,7 +348,7 @@ __global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64
     // phase 1: capacities and the CTA's sum
     unsigned long long mysum = 0;
     for (uint64_t v = v0 + threadIdx.x; v < v1; v += RB_THREADS) {
-        const uint32_t nc = cap_for(merged_len(g, b, vb, v), slack, min_cap);
+        const uint32_t nc = cap_for(merged_len<PK>(g, b, vb, v), slack, min_cap);
         vb.newcap[v] = nc;
         mysum += nc;
     }
@@ -382,7 +386,7 @@ __global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64
         if (v < v1) {
             const unsigned long long no = base + ex;
             vb.newoff[v] = no;
-            const Slab sl = g.slab[v];
+            const Slab sl = get_slab<PK>(g, v);
             big = vb.vseg[v] != NONE || sl.len > 16;
             if (!big) {
                 for (uint32_t j = 0; j < sl.len; j++) dst[no + j] = src[sl.off + j];
@@ -390,7 +394,7 @@ __global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64
                 ns.off = no;
                 ns.len = sl.len;
                 ns.cap = nc;
-                g.slab[v] = ns;
+                put_slab<PK>(g, v, ns);
             }
         }
         base += tot;
@@ -409,7 +413,7 @@ __global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64
     const uint64_t nwarps = ((uint64_t)gridDim.x * RB_THREADS) >> 5;
     for (uint64_t w = warp; w < nbig; w += nwarps) {
         const uint32_t v = __ldcg(&vb.big[w]);
-        const Slab sl = g.slab[v];
+        const Slab sl = get_slab<PK>(g, v);
         const unsigned long long no = __ldcg(&vb.newoff[v]);
         const uint32_t len = copy_merged_warp(src, dst, sl, no, kv, b, vb.vseg[v]);
         if (lane == 0) {
@@ -417,7 +421,7 @@ __global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64
             ns.off = no;
             ns.len = len;
             ns.cap = __ldcg(&vb.newcap[v]);
-            g.slab[v] = ns;
+            put_slab<PK>(g, v, ns);
         }
     }
     grid_sync(ctl);
@@ -434,6 +438,7 @@ __global__ void k_seg_cleanup(const uint64_t* __restrict__ kv, BatchBufs b,
 
 // ---------------------------------------------------------------- a2 restore
 
+template <bool PK>
 __global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t N, BatchBufs b,
                           uint32_t* __restrict__ touched, DevCtl* ctl) {
     if (*(volatile int*)&ctl->st.err != KERR_OK) return;
@@ -454,26 +459,25 @@ __global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t 
             }
         }
         if (!any) continue;
-        const int64_t dk = (int64_t)g.dout[u] + S0;  // post-batch d_out(u) (reading R3)
-        g.dout[u] = (uint32_t)dk;
+        const int64_t dk = (int64_t)*doutp<PK>(g, u) + S0;  // post-batch d_out(u) (reading R3)
+        *doutp<PK>(g, u) = (uint32_t)dk;
         for (uint32_t si = 0; si < g.S; si++) {
-            const size_t base = (size_t)si * g.n;
             double s1 = 0.0;
             for (uint64_t j = i0; j < i1; j++) {
                 if (!is_run_head(ku, j, i0)) continue;
                 const int32_t net = b.rnu[j];
-                if (net != 0) s1 += (double)net * g.P[base + (uint32_t)ku[j]];
+                if (net != 0) s1 += (double)net * *Pp<PK>(g, si, (uint32_t)ku[j]);
             }
             const double S1 = (1.0 - a) * s1;
             const double one = (u == g.sources[si]) ? 1.0 : 0.0;
-            const double pu = g.P[base + u];
-            const double r0 = g.R[base + u];
+            const double pu = *Pp<PK>(g, si, u);
+            const double r0 = *Rp<PK>(g, si, u);
             double r;
             if (dk > 0)
                 r = r0 + (S1 + (double)S0 * (a * one - pu - a * r0)) / (a * (double)dk);
             else
                 r = one - pu / a;  // Eq. 2 with an empty sum (reading R4)
-            g.R[base + u] = r;
+            *Rp<PK>(g, si, u) = r;
         }
         const unsigned pos = atomicAdd(&ctl->st.n_touched, 1u);
         touched[pos] = u;
@@ -482,30 +486,33 @@ __global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t 
 
 // ---------------------------------------------------------------- build / init / export
 
+template <bool PK>
 __global__ void k_build_count(const uint32_t* __restrict__ src, const uint32_t* __restrict__ dst,
                               uint64_t m, int undirected, DevGraph g) {
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
          i += (uint64_t)gridDim.x * blockDim.x) {
         const uint32_t u = src[i], v = dst[i];
-        atomicAdd(&g.slab[v].len, 1u);
-        atomicAdd(&g.dout[u], 1u);
+        atomicAdd(lenp<PK>(g, v), 1u);
+        atomicAdd(doutp<PK>(g, u), 1u);
         if (undirected && u != v) {
-            atomicAdd(&g.slab[u].len, 1u);
-            atomicAdd(&g.dout[v], 1u);
+            atomicAdd(lenp<PK>(g, u), 1u);
+            atomicAdd(doutp<PK>(g, v), 1u);
         }
     }
 }
 
+template <bool PK>
 __global__ void k_caps_from_len(DevGraph g, uint32_t* __restrict__ newcap, double slack,
                                 uint32_t min_cap) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x) {
-        const uint32_t len = g.slab[v].len;
+        const uint32_t len = *lenp<PK>(g, (uint32_t)v);
         uint32_t extra = (uint32_t)ceil((double)len * slack);
         newcap[v] = len + (extra > min_cap ? extra : min_cap);
     }
 }
 
+template <bool PK>
 __global__ void k_set_slabs(DevGraph g, const unsigned long long* __restrict__ off,
                             const uint32_t* __restrict__ cap) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
@@ -514,46 +521,66 @@ __global__ void k_set_slabs(DevGraph g, const unsigned long long* __restrict__ o
         s.off = off[v];
         s.len = 0;
         s.cap = cap[v];
-        g.slab[v] = s;
+        put_slab<PK>(g, v, s);
     }
 }
 
+template <bool PK>
 __global__ void k_build_fill(const uint32_t* __restrict__ src, const uint32_t* __restrict__ dst,
                              uint64_t m, int undirected, DevGraph g) {
     uint32_t* pool = g.pool[0];
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
          i += (uint64_t)gridDim.x * blockDim.x) {
         const uint32_t u = src[i], v = dst[i];
-        uint32_t p = atomicAdd(&g.slab[v].len, 1u);
-        pool[g.slab[v].off + p] = u;
+        uint32_t p = atomicAdd(lenp<PK>(g, v), 1u);
+        pool[get_slab<PK>(g, v).off + p] = u;
         if (undirected && u != v) {
-            p = atomicAdd(&g.slab[u].len, 1u);
-            pool[g.slab[u].off + p] = v;
+            p = atomicAdd(lenp<PK>(g, u), 1u);
+            pool[get_slab<PK>(g, u).off + p] = v;
         }
     }
 }
 
+template <bool PK>
 __global__ void k_init_state(DevGraph g) {
     // P = 0 and R = 0 are set by memset; R(s) = 1 for each source (Fig. 3 a(1))
     for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < g.S; i += gridDim.x * blockDim.x)
-        g.R[(size_t)i * g.n + g.sources[i]] = 1.0;
+        *Rp<PK>(g, i, g.sources[i]) = 1.0;
 }
 
+template <bool PK>
 __global__ void k_len_to_u32(DevGraph g, uint32_t* __restrict__ out) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x)
-        out[v] = g.slab[v].len;
+        out[v] = *lenp<PK>(g, (uint32_t)v);
 }
 
+template <bool PK>
 __global__ void k_export(DevGraph g, int active, const unsigned long long* __restrict__ off,
                          uint64_t* __restrict__ keys) {
     const uint32_t* pool = g.pool[active];
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x) {
-        const Slab sl = g.slab[v];
+        const Slab sl = get_slab<PK>(g, v);
         for (uint32_t j = 0; j < sl.len; j++) keys[off[v] + j] = (v << 32) | pool[sl.off + j];
     }
 }
+
+// packed layout: P, R, d_out out of the records (query / export / reset)
+__global__ void k_gather_rec(DevGraph g, double* __restrict__ P, double* __restrict__ R,
+                             uint32_t* __restrict__ dout, int zero_pr) {
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
+         v += (uint64_t)gridDim.x * blockDim.x) {
+        VRec* rc = &g.rec[v];
+        if (P) P[v] = rc->p;
+        if (R) R[v] = rc->r;
+        if (dout) dout[v] = rc->dout;
+        if (zero_pr) rc->p = rc->r = 0.0;
+    }
+}
+
+// the kernel instance for the handle's layout
+#define LAUNCH_PK(k) (g.rec ? k<true> : k<false>)
 
 inline unsigned grid_for(uint64_t n, unsigned threads, unsigned cap = 148 * 32) {
     uint64_t b = (n + threads - 1) / threads;
@@ -588,14 +615,14 @@ void launch_heads(const uint64_t* keys, const uint32_t* ops, uint64_t N, int32_t
 void launch_store_validate(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                            const VertexBufs& vb, DevCtl* ctl, int force_rebuild, cudaStream_t st,
                            uint32_t* launches) {
-    k_store_validate<<<grid_for(N * 32, 256), 256, 0, st>>>(g, kv, N, b, vb.vseg, ctl,
+    LAUNCH_PK(k_store_validate)<<<grid_for(N * 32, 256), 256, 0, st>>>(g, kv, N, b, vb.vseg, ctl,
                                                             force_rebuild);
     ++*launches;
 }
 
 void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                         DevCtl* ctl, cudaStream_t st, uint32_t* launches) {
-    k_store_apply<<<grid_for(N * 32, 256), 256, 0, st>>>(g, kv, b, ctl);
+    LAUNCH_PK(k_store_apply)<<<grid_for(N * 32, 256), 256, 0, st>>>(g, kv, b, ctl);
     ++*launches;
 }
 
@@ -608,7 +635,7 @@ void launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, con
         int per_sm = 0, sms = 0, dev = 0;
         cudaGetDevice(&dev);
         cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_rebuild, RB_THREADS, 0);
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_rebuild<false>, RB_THREADS, 0);
         grid = sms * (per_sm < 4 ? (per_sm < 1 ? 1 : per_sm) : 4);
     }
     DevGraph gg = g;
@@ -620,7 +647,8 @@ void launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, con
     uint64_t alt_cap = sp.alt_cap;
     DevCtl* c = ctl;
     void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &alt_cap, &c};
-    cudaLaunchCooperativeKernel((const void*)k_rebuild, dim3(grid), dim3(RB_THREADS), args, 0, st);
+    const void* fn = g.rec ? (const void*)k_rebuild<true> : (const void*)k_rebuild<false>;
+    cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(RB_THREADS), args, 0, st);
     ++*launches;
 }
 
@@ -632,44 +660,50 @@ void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, cons
 
 void launch_restore(const DevGraph& g, const uint64_t* ku, uint64_t N, const BatchBufs& b,
                     const VertexBufs& vb, DevCtl* ctl, cudaStream_t st, uint32_t* launches) {
-    k_restore<<<grid_for(N, 128), 128, 0, st>>>(g, ku, N, b, vb.touched, ctl);
+    LAUNCH_PK(k_restore)<<<grid_for(N, 128), 128, 0, st>>>(g, ku, N, b, vb.touched, ctl);
     ++*launches;
 }
 
 void launch_build_count(const uint32_t* src, const uint32_t* dst, uint64_t m, int undirected,
                         const DevGraph& g, uint32_t n, cudaStream_t st, uint32_t* launches) {
     (void)n;
-    k_build_count<<<grid_for(m, 256), 256, 0, st>>>(src, dst, m, undirected, g);
+    LAUNCH_PK(k_build_count)<<<grid_for(m, 256), 256, 0, st>>>(src, dst, m, undirected, g);
     ++*launches;
 }
 
 void launch_caps_from_len(const DevGraph& g, const VertexBufs& vb, double slack, uint32_t min_cap,
                           cudaStream_t st, uint32_t* launches) {
-    k_caps_from_len<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb.newcap, slack, min_cap);
+    LAUNCH_PK(k_caps_from_len)<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb.newcap, slack, min_cap);
     ++*launches;
 }
 
 void launch_build_fill(const uint32_t* src, const uint32_t* dst, uint64_t m, int undirected,
                        const DevGraph& g, const VertexBufs& vb, cudaStream_t st,
                        uint32_t* launches) {
-    k_set_slabs<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb.newoff, vb.newcap);
-    k_build_fill<<<grid_for(m, 256), 256, 0, st>>>(src, dst, m, undirected, g);
+    LAUNCH_PK(k_set_slabs)<<<grid_for(g.n, 256), 256, 0, st>>>(g, vb.newoff, vb.newcap);
+    LAUNCH_PK(k_build_fill)<<<grid_for(m, 256), 256, 0, st>>>(src, dst, m, undirected, g);
     *launches += 2;
 }
 
 void launch_init_state(const DevGraph& g, cudaStream_t st, uint32_t* launches) {
-    k_init_state<<<grid_for(g.S, 256), 256, 0, st>>>(g);
+    LAUNCH_PK(k_init_state)<<<grid_for(g.S, 256), 256, 0, st>>>(g);
     ++*launches;
 }
 
 void launch_export(const DevGraph& g, int active, const unsigned long long* off, uint64_t* keys,
                    cudaStream_t st, uint32_t* launches) {
-    k_export<<<grid_for(g.n, 256), 256, 0, st>>>(g, active, off, keys);
+    LAUNCH_PK(k_export)<<<grid_for(g.n, 256), 256, 0, st>>>(g, active, off, keys);
+    ++*launches;
+}
+
+void launch_gather_rec(const DevGraph& g, double* P, double* R, uint32_t* dout, int zero_pr,
+                       cudaStream_t st, uint32_t* launches) {
+    k_gather_rec<<<grid_for(g.n, 256), 256, 0, st>>>(g, P, R, dout, zero_pr);
     ++*launches;
 }
 
 void launch_len_to_u32(const DevGraph& g, uint32_t* out, cudaStream_t st, uint32_t* launches) {
-    k_len_to_u32<<<grid_for(g.n, 256), 256, 0, st>>>(g, out);
+    LAUNCH_PK(k_len_to_u32)<<<grid_for(g.n, 256), 256, 0, st>>>(g, out);
     ++*launches;
 }
 

@@ -219,7 +219,8 @@ def config_block(args, cfg, eps, S):
             "undirected": cfg["undirected"], "alpha": 0.15, "eps": eps,
             "source_band": f"top-{cfg['band']} out-degree", "sources": S,
             "rmat_abc": list(cfg["abc"]), "mode": args.mode,
-            "l2": "flushed between steps (512 MiB write)" if not args.no_flush else "not flushed"}
+            "l2": ("persisting lines reset + flushed between steps (512 MiB write)"
+                   if not args.no_flush else "not flushed")}
 
 
 # ---------------------------------------------------------------- our arm
@@ -304,6 +305,7 @@ def run_ours(args):
 
     def flush():
         if not args.no_flush:
+            ppr.reset_persisting_l2()  # the handle pins R/d_out in L2; unpin, then evict
             flush_buf.fill_(1)
 
     def bcast(t):

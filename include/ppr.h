@@ -158,6 +158,13 @@ enum {
 };
 ppr_status ppr_set_option(ppr_ctx *h, int key, int64_t value);
 
+/* Measurement utility: returns every persisting L2 line of the calling
+ * thread's current device to normal (evictable) status, so that a following
+ * L2 flush really empties the cache.  Handles keep their residual and
+ * out-degree arrays in a persisting L2 window;
+ * bench.py calls this before its between-step flush. */
+ppr_status ppr_reset_persisting_l2(void);
+
 /* Device memory held by the handle, in bytes. */
 uint64_t ppr_device_bytes(const ppr_ctx *h);
 

@@ -54,6 +54,7 @@ class BatchStats(ctypes.Structure):
 # every symbol include/ppr.h declares
 EXPORTS = ["ppr_create", "ppr_apply_batch", "ppr_push", "ppr_query", "ppr_export_edges",
            "ppr_export_dout", "ppr_set_option", "ppr_reset", "ppr_device_bytes", "ppr_destroy",
+           "ppr_reset_persisting_l2",
            "ppr_status_str", "ppr_last_error"]
 
 _lib = None
@@ -81,6 +82,8 @@ def load(path: str = LIB_PATH):
     lib.ppr_export_edges.argtypes = [vp, u32p, u32p, ctypes.c_uint64, ctypes.POINTER(ctypes.c_uint64)]
     lib.ppr_export_dout.argtypes = [vp, u32p]
     lib.ppr_set_option.argtypes = [vp, ctypes.c_int, ctypes.c_int64]
+    lib.ppr_reset_persisting_l2.argtypes = []
+    lib.ppr_reset_persisting_l2.restype = ctypes.c_int
     lib.ppr_device_bytes.argtypes = [vp]
     lib.ppr_device_bytes.restype = ctypes.c_uint64
     lib.ppr_destroy.argtypes = [vp]
@@ -93,6 +96,11 @@ def load(path: str = LIB_PATH):
         getattr(lib, f).restype = ctypes.c_int
     _lib = lib
     return lib
+
+
+def reset_persisting_l2():
+    """Return persisting L2 lines to normal status (call before an L2 flush)."""
+    return load().ppr_reset_persisting_l2()
 
 
 class PprError(RuntimeError):

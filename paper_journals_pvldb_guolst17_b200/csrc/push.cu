@@ -45,7 +45,13 @@ namespace {
 
 constexpr int PT = PUSH_THREADS;
 constexpr int NW = PT / 32;     // warps per CTA
-constexpr int U = 4;            // edges per lane per step
+#ifndef PPR_PUSH_OVERLAP
+#define PPR_PUSH_OVERLAP 1
+#endif
+#ifndef PPR_PUSH_U
+#define PPR_PUSH_U 2
+#endif
+constexpr int U = PPR_PUSH_U;   // edges per lane per step
 constexpr int QW = 256;         // per-warp queue slice (entries)
 enum { M_OPT = 0, M_EAGER = 1, M_DUP = 2, M_VAN = 3, M_ASYNC = 4 };
 // how a warp tile gets r and decides enqueues
@@ -124,7 +130,7 @@ __device__ __forceinline__ void ensure_room(Smem& s, Ctx& c, uint32_t need) {
 }
 
 // end of a round: all slices of the CTA go out with one global atomic
-__device__ void block_flush(Smem& s, Ctx& c) {
+__device__ __forceinline__ void block_flush(Smem& s, Ctx& c) {
     const unsigned w = warp();
     __syncwarp();
     if (lane() == 0) s.wq[w] = c.qn;
@@ -263,6 +269,35 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
 #pragma unroll
         for (int k = 0; k < U; k++)
             d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_pol(&a.g.dout[v[k]], pol_keep));
+#if PPR_PUSH_OVERLAP
+        // all U atomics are issued before any result is consumed, so the U
+        // chains overlap (the enqueues below synchronise the warp)
+        double incr[U], pre[U];
+        uint32_t sj[U];
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            if (j[k] >= 0) {
+                sj[k] = s.sid[j[k]];
+                incr[k] = __ddiv_rn(s.w[j[k]], (double)d[k]);
+                pre[k] = atom_add_pol(Rp<PK>(a.g, sj[k], v[k]), incr[k], pol_keep);
+            }
+        }
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            bool enq = false;
+            unsigned long long ev = 0;
+            if (j[k] >= 0) {
+                const double cur = __dadd_rn(pre[k], incr[k]);  // == the stored value (no FMA)
+                ev = ((unsigned long long)sj[k] << 32) | v[k];
+                if (KIND == K_OPT || KIND == K_DUP)
+                    enq = crossed<POS>(pre[k], cur, eps);   // Alg 4 line 16
+                else
+                    enq = push_cond<POS>(cur, eps) &&
+                          test_and_set(a.bitmap, (size_t)sj[k] * n + v[k]);  // UniqueEnqueue
+            }
+            warp_enqueue(s, c, enq, ev);
+        }
+#else
 #pragma unroll
         for (int k = 0; k < U; k++) {
             bool enq = false;
@@ -281,6 +316,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             }
             warp_enqueue(s, c, enq, ev);
         }
+#endif
     }
     if (KIND == K_OPT) {  // re-enqueue on the result of the fused self-update
         bool re = false;
@@ -296,7 +332,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
 // Every CTA takes tiles of T entries: its first tile statically, the rest by
 // one atomic claim each, until C is covered.
 template <bool POS, int KIND, bool PK>
-__device__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a, const unsigned long long* Fin,
+__device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a, const unsigned long long* Fin,
                               uint64_t C, unsigned long long* tc) {
     uint64_t per = (C + gridDim.x - 1) / gridDim.x;
     uint32_t T = (uint32_t)((per + 31) / 32 * 32);
@@ -323,7 +359,7 @@ __device__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a, const unsigned
 
 // self-update session of Alg 3 (lines 13-16): w = R(u), P(u) += a w, R(u) = 0
 template <bool PK>
-__device__ void session_snapshot(Ctx& c, const PushArgs& a, const unsigned long long* Fin,
+__device__ __forceinline__ void session_snapshot(Ctx& c, const PushArgs& a, const unsigned long long* Fin,
                                  uint64_t C, bool bitmap) {
     const double alpha = a.g.alpha;
     for (uint64_t idx = (uint64_t)blockIdx.x * PT + threadIdx.x; idx < C;
@@ -343,7 +379,7 @@ __device__ void session_snapshot(Ctx& c, const PushArgs& a, const unsigned long 
 
 // Eager: self-update with the r_u recorded during propagation (Alg 4 lines 19-23)
 template <bool POS, bool PK>
-__device__ void session_eager_self(Smem& s, Ctx& c, const PushArgs& a,
+__device__ __forceinline__ void session_eager_self(Smem& s, Ctx& c, const PushArgs& a,
                                    const unsigned long long* Fin, uint64_t C) {
     const double eps = a.g.eps, alpha = a.g.alpha;
     const uint64_t stride = (uint64_t)gridDim.x * PT;
@@ -368,7 +404,7 @@ __device__ void session_eager_self(Smem& s, Ctx& c, const PushArgs& a,
     }
 }
 
-__device__ void clear_frontier_bits(Ctx& c, const PushArgs& a, const unsigned long long* Fin,
+__device__ __forceinline__ void clear_frontier_bits(Ctx& c, const PushArgs& a, const unsigned long long* Fin,
                                     uint64_t C) {
     for (uint64_t idx = (uint64_t)blockIdx.x * PT + threadIdx.x; idx < C;
          idx += (uint64_t)gridDim.x * PT) {
@@ -380,7 +416,7 @@ __device__ void clear_frontier_bits(Ctx& c, const PushArgs& a, const unsigned lo
 // ---------------------------------------------------------------- seeding
 
 template <bool POS, bool PK>
-__device__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
+__device__ __forceinline__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
     const double eps = a.g.eps;
     const uint64_t stride = (uint64_t)gridDim.x * PT;
     uint64_t total;
@@ -419,7 +455,7 @@ __device__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
 // ---------------------------------------------------------------- phase driver
 
 template <int MODE, bool POS, bool PK>
-__device__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
+__device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
     DevCtl* ctl = a.ctl;
     const int ph = POS ? 0 : 1;
     // seed into F[it%2] / fcount[it%3]; both that and the next counter are 0 here
@@ -556,7 +592,7 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
 // reading done == tail (done first) means no entry is queued or in progress.
 
 template <bool POS, bool PK>
-__device__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
+__device__ __forceinline__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
     DevCtl* ctl = a.ctl;
     unsigned long long* head = &ctl->tilectr[0].v;
     unsigned long long* tail = &ctl->fcount[0].v;

@@ -7,8 +7,14 @@
 
 namespace ppr {
 
-constexpr int PUSH_THREADS = 256;   // one frontier tile = up to PUSH_THREADS entries
-constexpr int PUSH_MIN_BLOCKS = 4;  // resident CTAs per SM (persistent grid = SMs x this)
+#ifndef PPR_PUSH_THREADS
+#define PPR_PUSH_THREADS 256
+#endif
+constexpr int PUSH_THREADS = PPR_PUSH_THREADS;  // one frontier tile = up to PUSH_THREADS entries
+#ifndef PPR_PUSH_MIN_BLOCKS
+#define PPR_PUSH_MIN_BLOCKS 4
+#endif
+constexpr int PUSH_MIN_BLOCKS = PPR_PUSH_MIN_BLOCKS;  // resident CTAs per SM (persistent grid = SMs x this)
 
 struct PushArgs {
     DevGraph g;

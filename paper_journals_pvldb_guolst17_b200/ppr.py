@@ -60,7 +60,7 @@ EXPORTS = ["ppr_create", "ppr_apply_batch", "ppr_push", "ppr_query", "ppr_export
 _lib = None
 
 
-def load(path: str = LIB_PATH):
+def load(path: str = os.environ.get("PPR_LIB", LIB_PATH)):
     """Loads libppr.so (fails loudly if it has not been built)."""
     global _lib
     if _lib is not None:

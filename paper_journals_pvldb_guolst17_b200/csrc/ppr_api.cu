@@ -56,6 +56,8 @@ struct ppr_ctx {
     double* d_hot = nullptr;     // arrays layout: R [S][n] followed by d_out [n] (one allocation,
     uint64_t hot_bytes = 0;      //   the L2 access-policy window / persisting set-aside)
     bool l2_window = false;
+    size_t l2_win_bytes = 0;
+    float l2_hit = 0.f;
     uint32_t* d_dout = nullptr;  // structure-of-arrays layout (S > 1)
     Slab* d_slab = nullptr;
     uint32_t* d_pool[2] = {nullptr, nullptr};
@@ -263,6 +265,9 @@ PushArgs push_args(ppr_ctx* h) {
     a.phases = 3;
     a.max_iters = h->max_iters;
     a.iter_cap = 1000000;
+    a.l2_base = h->d_hot;
+    a.l2_bytes = h->l2_win_bytes;
+    a.l2_hit = h->l2_hit;
     if (h->d_trace) {
         cudaMemsetAsync(h->d_trace, 0, sizeof(unsigned long long) * (4 * h->trace_cap + 8), h->st);
         a.trace = h->d_trace;
@@ -511,6 +516,8 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
                 av.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
                 h->l2_window =
                     cudaStreamSetAttribute(h->st, cudaStreamAttributeAccessPolicyWindow, &av) == cudaSuccess;
+                h->l2_win_bytes = win;
+                h->l2_hit = av.accessPolicyWindow.hitRatio;
                 cudaGetLastError();
             }
         }

@@ -576,6 +576,33 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
     }
 }
 
+// cooperative launch carrying the L2 access-policy window as a launch attribute
+inline cudaError_t coop_launch(const void* fn, int grid, const PushArgs& a, cudaStream_t st) {
+    PushArgs copy = a;
+    void* args[] = {&copy};
+    cudaLaunchConfig_t cfg{};
+    cfg.gridDim = dim3(grid);
+    cfg.blockDim = dim3(PT);
+    cfg.stream = st;
+    cudaLaunchAttribute at[2];
+    int na = 0;
+    at[na].id = cudaLaunchAttributeCooperative;
+    at[na].val.cooperative = 1;
+    na++;
+    if (a.l2_bytes) {
+        at[na].id = cudaLaunchAttributeAccessPolicyWindow;
+        at[na].val.accessPolicyWindow.base_ptr = a.l2_base;
+        at[na].val.accessPolicyWindow.num_bytes = a.l2_bytes;
+        at[na].val.accessPolicyWindow.hitRatio = a.l2_hit;
+        at[na].val.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
+        at[na].val.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
+        na++;
+    }
+    cfg.attrs = at;
+    cfg.numAttrs = na;
+    return cudaLaunchKernelExC(&cfg, fn, args);
+}
+
 // ---------------------------------------------------------------- asynchronous schedule
 //
 // PPR_MODE_ASYNC: the same Alg 4 operations on every frontier vertex (eager
@@ -711,10 +738,7 @@ cudaError_t launch_async(const PushArgs& a, int num_sms, cudaStream_t st) {
         if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
         if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
     }
-    dim3 grid(num_sms * blocks_per_sm), block(PT);
-    PushArgs copy = a;
-    void* args[] = {&copy};
-    return cudaLaunchCooperativeKernel((const void*)k_push_async<PK>, grid, block, args, 0, st);
+    return coop_launch((const void*)k_push_async<PK>, num_sms * blocks_per_sm, a, st);
 }
 
 template <int MODE, bool PK>
@@ -727,10 +751,7 @@ cudaError_t launch_mode(const PushArgs& a, int num_sms, cudaStream_t st) {
         if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
         if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
     }
-    dim3 grid(num_sms * blocks_per_sm), block(PT);
-    PushArgs copy = a;
-    void* args[] = {&copy};
-    return cudaLaunchCooperativeKernel((const void*)k_push<MODE, PK>, grid, block, args, 0, st);
+    return coop_launch((const void*)k_push<MODE, PK>, num_sms * blocks_per_sm, a, st);
 }
 
 template <bool PK>

@@ -18,6 +18,9 @@ constexpr int PUSH_MIN_BLOCKS = PPR_PUSH_MIN_BLOCKS;  // resident CTAs per SM (p
 
 struct PushArgs {
     DevGraph g;
+    void* l2_base;             // persisting L2 window (R and d_out), l2_bytes = 0: none
+    size_t l2_bytes;
+    float l2_hit;
     DevCtl* ctl;
     unsigned long long* F[2];  // frontier buffers, capacity S*n each
     double* W;                 // Alg 3 snapshot / Alg 4 r_u, aligned with F

@@ -229,7 +229,7 @@ def run_ours(args):
     import torch
     import torch.distributed as dist
 
-    from paper_journals_pvldb_guolst17_b200 import ppr, workload as W
+    from paper_journals_pvldb_guolst17_b200 import dist as D, ppr, workload as W
 
     ws, rank, local = dist_env()
     if ws > 1:
@@ -248,27 +248,41 @@ def run_ours(args):
     cfg.update(over)
     eps = args.eps or cfg["eps"]
     S = args.sources or ws
-    if S % ws:
-        raise SystemExit("--sources must be a multiple of the world size")
+    if S < ws:
+        raise SystemExit("--sources must be >= the world size")
     steps, warm = args.steps, max(args.warmup, 3)
     nslides = steps * (1 if args.no_e2e else 2) + warm
+    und = bool(cfg["undirected"])
+    nI, nD = cfg["ins"], cfg["dele"]  # per slide, as given (undirected: edges)
 
-    # rank 0 owns the stream; the window and the batches go to the other
-    # ranks over NCCL (setup: untimed; per-batch broadcast: timed)
+    # rank 0 owns the stream; the window, the sources and every batch reach the
+    # other ranks over NCCL (setup untimed; the per-batch broadcast is timed)
+    t0 = time.perf_counter()
     if rank == 0:
         st, cfg = W.make_stream(args.workload, seed=args.seed, **over)
-        g0s, g0d = st.window()
-        srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], S)
-        batches = [st.next_batch() for _ in range(nslides)]
+        g0s, g0d = (st.src[st.lo:st.hi].copy(), st.dst[st.lo:st.hi].copy()) if und else st.window()
+        arcs_s, arcs_d = W.expand_undirected(g0s, g0d) if und else (g0s, g0d)
+        srcs = W.pick_sources(cfg["n"], arcs_s, arcs_d, cfg["band"], S)
+        batches = []
+        for _ in range(nslides):
+            i0, i1 = st.hi, st.hi + nI
+            d0, d1 = st.lo, st.lo + nD
+            if und:  # the library expands undirected edges itself
+                b = (st.src[i0:i1], st.dst[i0:i1], st.src[d0:d1], st.dst[d0:d1])
+                st.hi, st.lo = i1, d1
+            else:
+                b = st.next_batch()
+            batches.append(tuple(np.ascontiguousarray(x) for x in b))
         meta = torch.tensor([len(g0s)], dtype=torch.int64, device=dev)
     else:
         meta = torch.zeros(1, dtype=torch.int64, device=dev)
+    t_gen = time.perf_counter() - t0
     if ws > 1:
         dist.broadcast(meta, 0)
     m0 = int(meta.item())
     if rank == 0:
-        win = torch.from_numpy(np.stack([g0s, g0d]).astype(np.int32)).to(dev)
-        srct = torch.from_numpy(srcs.astype(np.int32)).to(dev)
+        win = torch.from_numpy(np.stack([g0s, g0d]).view(np.int32)).to(dev)
+        srct = torch.from_numpy(srcs.view(np.int32)).to(dev)
     else:
         win = torch.empty((2, m0), dtype=torch.int32, device=dev)
         srct = torch.empty(S, dtype=torch.int32, device=dev)
@@ -277,30 +291,26 @@ def run_ours(args):
         dist.broadcast(srct, 0)
     win_np = win.cpu().numpy().view(np.uint32)
     srcs_all = srct.cpu().numpy().view(np.uint32)
-    per_rank = S // ws
-    my_srcs = srcs_all[rank * per_rank:(rank + 1) * per_rank]
-    nI, nD = cfg["ins"], cfg["dele"]
-    if cfg["undirected"]:
-        raise SystemExit("undirected workloads: expand on rank 0 (not wired in bench yet)")
+    del win
+    deg = np.bincount(win_np[0], minlength=cfg["n"])
+    if und:
+        deg = deg + np.bincount(win_np[1], minlength=cfg["n"])
+    my_srcs = D.partition_sources(srcs_all, deg, ws, rank)
 
     t0 = time.perf_counter()
     h = ppr.Ppr(cfg["n"], win_np[0], win_np[1], my_srcs, alpha=0.15, eps=eps, mode=args.mode,
-                device=local, stream=ctypes_stream(stream))
+                device=local, stream=ctypes_stream(stream), undirected=und)
+    torch.cuda.synchronize()
     t_create = time.perf_counter() - t0
     create_stats = h.create_stats
-    del win, win_np
+    del win_np
 
-    # device-resident batches (rank 0) packed as [4, n]: ins_src, ins_dst, del_src, del_dst
-    def pack(b):
-        return torch.from_numpy(np.stack([b[0], b[1], b[2], b[3]]).astype(np.int32))
-
-    dev_batches = []
+    counts = (nI, nD)
+    nflat = 2 * (nI + nD)
     if rank == 0:
-        for b in batches[:warm + steps]:
-            dev_batches.append(pack(b).to(dev))
+        dev_batches = [D.pack_batch(*b)[0].to(dev) for b in batches[:warm + steps]]
     else:
-        for _ in range(warm + steps):
-            dev_batches.append(torch.empty((4, nI), dtype=torch.int32, device=dev))
+        dev_batches = [torch.empty(nflat, dtype=torch.int32, device=dev) for _ in range(warm + steps)]
     flush_buf = torch.empty(512 * 1024 * 1024 // 4, dtype=torch.int32, device=dev)
 
     def flush():
@@ -308,18 +318,12 @@ def run_ours(args):
             ppr.reset_persisting_l2()  # the handle pins R/d_out in L2; unpin, then evict
             flush_buf.fill_(1)
 
-    def bcast(t):
-        if ws > 1:
-            dist.broadcast(t, 0)
+    def step_device(flat):
+        flat = D.broadcast_batch(flat, counts)
+        return h.apply_batch(*D.unpack_batch(flat, counts), mem=ppr.MEM_DEVICE)
 
-    def step_device(t):
-        bt = dev_batches[t]
-        bcast(bt)
-        return h.apply_batch(bt[0], bt[1], bt[2], bt[3], mem=ppr.MEM_DEVICE)
-
-    # warm-up
     for t in range(warm):
-        step_device(t)
+        step_device(dev_batches[t])
     torch.cuda.synchronize()
     if ws > 1:
         dist.barrier()
@@ -336,7 +340,7 @@ def run_ours(args):
     for k in range(steps):
         flush()
         ev[k][0].record(stream)
-        stats.append(step_device(warm + k))
+        stats.append(step_device(dev_batches[warm + k]))
         ev[k][1].record(stream)
     torch.cuda.synchronize()
     if ws > 1:
@@ -344,27 +348,24 @@ def run_ours(args):
     ms = [a.elapsed_time(b) for a, b in ev]
 
     # timed: end to end from pinned host buffers through the same call
-    e2e_ms = []
-    e2e_stats = []
+    e2e_ms, e2e_stats = [], []
     if not args.no_e2e:
         host = []
         if rank == 0:
-            for b in batches[warm + steps:warm + 2 * steps]:
-                host.append(pack(b).pin_memory())
+            host = [D.pack_batch(*b)[0].pin_memory() for b in batches[warm + steps:warm + 2 * steps]]
+        buf = torch.empty(nflat, dtype=torch.int32, device=dev)
         for k in range(steps):
             flush()
             a_, b_ = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
             a_.record(stream)
             if ws > 1:
-                buf = dev_batches[k]
                 if rank == 0:
                     buf.copy_(host[k], non_blocking=True)
-                bcast(buf)
-                s_ = h.apply_batch(buf[0], buf[1], buf[2], buf[3], mem=ppr.MEM_DEVICE)
-                s_["h2d_bytes"] = 16 * nI if rank == 0 else 0
+                s_ = step_device(buf)
+                s_["h2d_bytes"] = 4 * nflat if rank == 0 else 0
             else:
-                hb = host[k].numpy()
-                s_ = h.apply_batch(hb[0], hb[1], hb[2], hb[3], mem=ppr.MEM_HOST)
+                hb = host[k].numpy().view(np.uint32)
+                s_ = h.apply_batch(*D.unpack_batch(hb, counts), mem=ppr.MEM_HOST)
             b_.record(stream)
             b_.synchronize()
             e2e_ms.append(a_.elapsed_time(b_))
@@ -372,23 +373,21 @@ def run_ours(args):
         torch.cuda.synchronize()
     clk = clocks.stop()
 
-    # max over ranks of the summed step time
-    T = sum(ms)
-    T_e2e = sum(e2e_ms) if e2e_ms else 0.0
+    # post-run validity: termination (-eps <= R <= eps) for this rank's first source
+    P0, R0 = h.query(0)
+    term_ok = bool(np.all(np.abs(R0) <= eps))
+    term_ok = D.max_over_ranks(0.0 if term_ok else 1.0, device=dev) == 0.0
+
+    T = D.max_over_ranks(sum(ms), device=dev)
+    T_e2e = D.max_over_ranks(sum(e2e_ms), device=dev) if e2e_ms else 0.0
     push_ms = sum(s["ms_push"] for s in stats)
-    edges = sum(s["pushed_edges"] for s in stats)
-    verts = sum(s["pushes"] for s in stats)
-    launches = sum(s["kernel_launches"] for s in stats)
-    vec = torch.tensor([T, T_e2e, push_ms, edges, verts, launches], dtype=torch.float64, device=dev)
-    if ws > 1:
-        tmax = torch.tensor([T, T_e2e], dtype=torch.float64, device=dev)
-        dist.all_reduce(tmax, op=dist.ReduceOp.MAX)
-        tot = vec.clone()
-        dist.all_reduce(tot, op=dist.ReduceOp.SUM)
-        T, T_e2e = float(tmax[0]), float(tmax[1])
-        edges, verts, launches = float(tot[3]), float(tot[4]), float(tot[5])
+    edges_r0 = sum(s["pushed_edges"] for s in stats)
+    verts_r0 = sum(s["pushes"] for s in stats)
+    edges, verts, launches = D.sum_over_ranks(
+        [edges_r0, verts_r0, sum(s["kernel_launches"] for s in stats)], device=dev)
+    dev_bytes = h.device_bytes
+    h.close()
     if rank != 0:
-        h.close()
         if ws > 1:
             dist.destroy_process_group()
         return
@@ -397,30 +396,31 @@ def run_ours(args):
     value = S * upd * steps / (T / 1e3)
     e2e_value = S * upd * len(e2e_ms) / (T_e2e / 1e3) if e2e_ms else None
     peak, peak_kind = measured_peak()
-    # dominant kernel: the persistent push (one launch per step); rank 0's own launches
-    r0_edges = sum(s["pushed_edges"] for s in stats)
-    r0_verts = sum(s["pushes"] for s in stats)
-    bytes_per_launch = (B_EDGE * r0_edges + B_VERTEX * r0_verts) / steps
+    # dominant kernel: the persistent push (one launch per step), rank 0's launches
+    bytes_per_launch = (B_EDGE * edges_r0 + B_VERTEX * verts_r0) / steps
     push_ms_avg = push_ms / steps
     achieved = bytes_per_launch / (push_ms_avg / 1e3) / 1e9 if push_ms_avg > 0 else 0.0
-    traffic = profile_traffic(args.workload)
+    traffic = profile_traffic(args.workload) if S == 1 else None
 
     line = {
-        "metric": "edge updates/s", "value": value, "unit": "edge updates/s",
+        "metric": "edge updates/s", "value": value,
+        "unit": "edge updates/s" if S == 1 else "source-edge updates/s (S sources x updates)",
         "n_gpus": ws, "steps": steps, "warmup": warm, "ms_per_step": T / steps,
-        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64",
-        "data": "synthetic", "config": config_block(args, cfg, eps, S),
-        "e2e": ({"value": e2e_value, "unit": "edge updates/s",
+        "higher_is_better": True, "scaling": "weak" if not args.sources else "strong",
+        "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": config_block(args, cfg, eps, S),
+        "e2e": ({"value": e2e_value, "unit": "edge updates/s" if S == 1 else "source-edge updates/s",
                  "h2d_bytes_per_step": int(np.mean([s["h2d_bytes"] for s in e2e_stats])),
                  "d2h_bytes_per_step": int(np.mean([s["d2h_bytes"] for s in e2e_stats])),
                  "ms_per_step": T_e2e / len(e2e_ms)} if e2e_ms else None),
         "gpu_launches": int(launches),
         "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                      "frac": achieved / peak, "traffic": traffic,
-                     "kernel": "k_push<OPT> (persistent, 1 launch/step)",
+                     "kernel": f"k_push<{args.mode.upper()}> (persistent, 1 launch/step)",
                      "algorithmic_bytes_per_launch": bytes_per_launch,
                      "peak_kind": peak_kind, "ms_per_launch": push_ms_avg},
         "clocks": clk,
+        "checks": {"termination_all_ranks": term_ok},
         "detail": {
             "ms_per_step_p50": statistics.median(ms), "ms_per_step_p95": float(np.percentile(ms, 95)),
             "ms_store": sum(s["ms_store"] for s in stats) / steps,
@@ -431,13 +431,16 @@ def run_ours(args):
             "pushed_edges_per_step": edges / steps / S,
             "iters_per_step": sum(s["iters_pos"] + s["iters_neg"] for s in stats) / steps,
             "rebuilds": sum(s["rebuilt"] for s in stats),
-            "create_s": t_create, "create_stats": create_stats,
-            "device_bytes": h.device_bytes,
+            "atomics_per_s_rank0": (edges_r0 + verts_r0) / (push_ms / 1e3) if push_ms else None,
+            "generate_s": t_gen, "create_s": t_create, "create_stats": create_stats,
+            "device_bytes_rank0": dev_bytes, "sources_per_rank": len(my_srcs),
         },
     }
     if not args.no_cpu_baseline and ws == 1:
-        line["cpu_baseline"] = cpu_baseline(args, cfg, eps, my_srcs[:1], g0s, g0d, batches)
-    h.close()
+        arcs = (W.expand_undirected(g0s, g0d) if und else (g0s, g0d))
+        bl = [(W.expand_undirected(b[0], b[1]) + W.expand_undirected(b[2], b[3])) if und else b
+              for b in batches]
+        line["cpu_baseline"] = cpu_baseline(args, cfg, eps, my_srcs[:1], arcs[0], arcs[1], bl)
     print(json.dumps(line), flush=True)
     if ws > 1:
         dist.destroy_process_group()

@@ -822,6 +822,23 @@ ppr_status ppr_query(ppr_ctx* h, uint32_t source_idx, double* P_out, double* R_o
         if (e != cudaSuccess) return cuda_fail(h, e, "ppr_query");
         return PPR_OK;
     }
+    if (h->S > 1) {  // vertex-major [n][S]: gather the column through a device buffer
+        double* tmp = nullptr;
+        const bool host = mem == PPR_MEM_HOST;
+        if (host && dalloc(h, &tmp, h->n) != cudaSuccess) return PPR_ENOMEM;
+        uint32_t launches = 0;
+        const double* srcs[2] = {h->d_P, h->d_R};
+        double* outs[2] = {P_out, R_out};
+        for (int q = 0; q < 2 && e == cudaSuccess; q++) {
+            if (!outs[q]) continue;
+            launch_gather_col(srcs[q], h->S, source_idx, h->n, host ? tmp : outs[q], h->st, &launches);
+            if (host) e = cudaMemcpyAsync(outs[q], tmp, sizeof(double) * h->n, k, h->st);
+            if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
+        }
+        dfree(h, tmp, h->n);
+        if (e != cudaSuccess) return cuda_fail(h, e, "ppr_query");
+        return PPR_OK;
+    }
     if (P_out) e = cudaMemcpyAsync(P_out, h->d_P + off, sizeof(double) * h->n, k, h->st);
     if (e == cudaSuccess && R_out) e = cudaMemcpyAsync(R_out, h->d_R + off, sizeof(double) * h->n, k, h->st);
     if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);

@@ -90,17 +90,18 @@ struct DevGraph {
 };
 
 // ------------------------------------------------------------------ layout accessors
-// PK = packed (VRec) layout; otherwise structure of arrays with R, P as [S][n].
+// PK = packed (VRec) layout; otherwise arrays with R, P vertex-major [n][S] (the S
+// residuals of a vertex share cache lines; identical to [S][n] for S = 1).
 
 template <bool PK>
 __device__ __forceinline__ double* Rp(const DevGraph& g, uint32_t sidx, uint32_t v) {
     if (PK) return &g.rec[v].r;
-    return g.R + (size_t)sidx * g.n + v;
+    return g.R + (size_t)v * g.S + sidx;  // vertex-major [n][S]
 }
 template <bool PK>
 __device__ __forceinline__ double* Pp(const DevGraph& g, uint32_t sidx, uint32_t v) {
     if (PK) return &g.rec[v].p;
-    return g.P + (size_t)sidx * g.n + v;
+    return g.P + (size_t)v * g.S + sidx;
 }
 template <bool PK>
 __device__ __forceinline__ uint32_t* doutp(const DevGraph& g, uint32_t v) {

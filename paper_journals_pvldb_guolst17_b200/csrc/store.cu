@@ -579,6 +579,14 @@ __global__ void k_gather_rec(DevGraph g, double* __restrict__ P, double* __restr
     }
 }
 
+// arrays layout, S > 1: column `sidx` of a vertex-major [n][S] array
+__global__ void k_gather_col(const double* __restrict__ src, uint32_t S, uint32_t sidx, uint32_t n,
+                             double* __restrict__ dst) {
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
+         v += (uint64_t)gridDim.x * blockDim.x)
+        dst[v] = src[v * S + sidx];
+}
+
 // the kernel instance for the handle's layout
 #define LAUNCH_PK(k) (g.rec ? k<true> : k<false>)
 
@@ -699,6 +707,12 @@ void launch_export(const DevGraph& g, int active, const unsigned long long* off,
 void launch_gather_rec(const DevGraph& g, double* P, double* R, uint32_t* dout, int zero_pr,
                        cudaStream_t st, uint32_t* launches) {
     k_gather_rec<<<grid_for(g.n, 256), 256, 0, st>>>(g, P, R, dout, zero_pr);
+    ++*launches;
+}
+
+void launch_gather_col(const double* src, uint32_t S, uint32_t sidx, uint32_t n, double* dst,
+                       cudaStream_t st, uint32_t* launches) {
+    k_gather_col<<<grid_for(n, 256), 256, 0, st>>>(src, S, sidx, n, dst);
     ++*launches;
 }
 

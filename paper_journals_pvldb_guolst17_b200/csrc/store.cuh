@@ -88,6 +88,9 @@ void launch_init_state(const DevGraph& g, cudaStream_t st, uint32_t* launches);
 void launch_export(const DevGraph& g, int active, const unsigned long long* off, uint64_t* keys,
                    cudaStream_t st, uint32_t* launches);
 void launch_len_to_u32(const DevGraph& g, uint32_t* out, cudaStream_t st, uint32_t* launches);
+// arrays layout: dst[v] = src[v * S + sidx]
+void launch_gather_col(const double* src, uint32_t S, uint32_t sidx, uint32_t n, double* dst,
+                       cudaStream_t st, uint32_t* launches);
 // packed layout: copy P / R / d_out (any may be null) out of the records; zero_pr clears P and R
 void launch_gather_rec(const DevGraph& g, double* P, double* R, uint32_t* dout, int zero_pr,
                        cudaStream_t st, uint32_t* launches);

@@ -69,9 +69,13 @@ enum {
     PPR_MODE_EAGER = 1,     /* eager propagation, UniqueEnqueue via bitmap */
     PPR_MODE_DUPDETECT = 2, /* Alg 3 sessions + local duplicate detection */
     PPR_MODE_VANILLA = 3,   /* Alg 3 as printed: snapshot, barrier, propagate, UniqueEnqueue */
-    PPR_MODE_ASYNC = 4      /* Alg 4's operations without rounds: asynchronous ring worklist
+    PPR_MODE_ASYNC = 4,     /* Alg 4's operations without rounds: asynchronous ring worklist
                                (any push order is valid by Lemma 1; DESIGN.md K-ASYNC);
                                iters_pos/iters_neg are reported as 0 */
+    PPR_MODE_EAGER_SCAN = 5 /* eager propagation; residual updates are fire-and-forget
+                               reductions that mark touched vertices in a bitmap, and each
+                               round's frontier comes from a warp-ballot/scan compaction of
+                               that bitmap (DESIGN.md K-SCAN) */
 };
 
 /* Graph for ppr_create: m arcs src[i] -> dst[i] on [0, n) (host pointers).

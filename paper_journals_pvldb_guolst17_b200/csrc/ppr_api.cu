@@ -439,7 +439,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     o.slack = 0.25;
     o.min_cap = 4;
     if (opts) o = *opts;
-    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_ASYNC || !(o.slack >= 0.0) ||
+    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_EAGER_SCAN || !(o.slack >= 0.0) ||
         o.min_cap == 0)
         return PPR_EINVAL;
 
@@ -663,7 +663,7 @@ ppr_status ppr_set_option(ppr_ctx* h, int key, int64_t value) {
     if (h->poisoned) return PPR_EPOISONED;
     switch (key) {
         case PPR_OPT_MODE:
-            if (value < PPR_MODE_OPT || value > PPR_MODE_ASYNC) return PPR_EINVAL;
+            if (value < PPR_MODE_OPT || value > PPR_MODE_EAGER_SCAN) return PPR_EINVAL;
             h->mode = (int)value;
             return PPR_OK;
         case PPR_OPT_PUSH: h->push_enabled = value != 0; return PPR_OK;

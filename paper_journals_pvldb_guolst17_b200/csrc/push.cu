@@ -48,14 +48,20 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_PUSH_OVERLAP
 #define PPR_PUSH_OVERLAP 1
 #endif
+#ifndef PPR_PUSH_DYN
+#define PPR_PUSH_DYN 1
+#endif
 #ifndef PPR_PUSH_U
 #define PPR_PUSH_U 2
 #endif
 constexpr int U = PPR_PUSH_U;   // edges per lane per step
 constexpr int QW = 256;         // per-warp queue slice (entries)
-enum { M_OPT = 0, M_EAGER = 1, M_DUP = 2, M_VAN = 3, M_ASYNC = 4 };
+enum { M_OPT = 0, M_EAGER = 1, M_DUP = 2, M_VAN = 3, M_ASYNC = 4, M_SCAN = 5 };
 // how a warp tile gets r and decides enqueues
-enum { K_OPT = 0, K_EAGER = 1, K_DUP = 2, K_VAN = 3 };
+enum { K_OPT = 0, K_EAGER = 1, K_DUP = 2, K_VAN = 3, K_SCAN = 4 };
+// K_SCAN (mode EAGER_SCAN): eager read as in Opt, but every residual change is a
+// fire-and-forget reduction that also marks the touched vertex in a bitmap;
+// the next frontier is decided after a grid barrier by scanning the bitmap.
 
 struct Smem {
     uint32_t scan[PT + 1];                // exclusive in-degree prefix of the tile
@@ -67,6 +73,7 @@ struct Smem {
     unsigned long long gbase;
     unsigned long long next;              // next claimed tile
     unsigned long long cround;            // this round's frontier size
+    unsigned int chunk;                   // next 32-edge chunk of the tile (dynamic claims)
     uint32_t warp_tmp[NW + 1];            // block-scan scratch
 };
 
@@ -157,6 +164,10 @@ __device__ __forceinline__ bool test_and_set(uint32_t* bitmap, unsigned long lon
     return (old & mask) == 0;
 }
 
+__device__ __forceinline__ void mark_bit(uint32_t* bitmap, unsigned long long bit) {
+    atomicOr(&bitmap[bit >> 5], 1u << (bit & 31u));  // result unused: RED.OR
+}
+
 __device__ __forceinline__ void clear_bit(uint32_t* bitmap, unsigned long long bit) {
     atomicAnd(&bitmap[bit >> 5], ~(1u << (bit & 31u)));
 }
@@ -201,7 +212,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     double* ru = Rp<PK>(a.g, sidx, u);
     double r = 0.0;
     bool push = false;
-    if (KIND == K_OPT || KIND == K_EAGER) {
+    if (KIND == K_OPT || KIND == K_EAGER || KIND == K_SCAN) {
         r = valid ? ld_relaxed_f64(ru) : 0.0;  // Alg 4 line 10: the current R(u)
         // A queued vertex meets pushCond (it was enqueued on a crossing, and R(u)
         // only grows until its own self-update).  If the relaxed load returned
@@ -223,6 +234,12 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
         self_old = atomicAdd(ru, -r);
         red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
     }
+    if (KIND == K_SCAN && push) {  // self-update: no result needed; u is re-tested at the scan
+        red_add_pol(ru, -r, l2_keep());
+        red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
+        mark_bit(a.bitmap, (size_t)u * a.g.S + sidx);
+        c.pushes++;
+    }
     uint32_t len = 0;
     unsigned long long off = 0;
     if (push) {
@@ -239,7 +256,10 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     uint32_t E;
     const uint32_t ex = block_exclusive_scan_u32<PT>(len, s.warp_tmp, &E);
     s.scan[threadIdx.x] = threadIdx.x < T ? ex : 0xFFFFFFFFu;
-    if (threadIdx.x == 0) s.scan[PT] = 0xFFFFFFFFu;
+    if (threadIdx.x == 0) {
+        s.scan[PT] = 0xFFFFFFFFu;
+        s.chunk = 0;
+    }
     s.off[threadIdx.x] = off;
     s.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
     s.sid[threadIdx.x] = sidx;
@@ -251,13 +271,53 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     }
     const unsigned long long pol_keep = l2_keep(), pol_stream = l2_stream();
     // 32-edge chunks dealt round-robin to the warps (chunk w + NW*i), U per step
+    if (KIND == K_SCAN) {  // fire-and-forget edge walk: no enqueue decisions here
+        for (uint32_t cb = w; cb * 32 < E; cb += NW * U) {
+            uint32_t v[U], d[U];
+            int j[U];
+#pragma unroll
+            for (int k = 0; k < U; k++) {
+                const uint32_t e = (cb + NW * k) * 32 + L;
+                j[k] = -1;
+                v[k] = 0;
+                if (e < E) {
+                    j[k] = owner_of(s.scan, e, top);
+                    v[k] = ld_u32_pol(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
+                }
+            }
+#pragma unroll
+            for (int k = 0; k < U; k++)
+                d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_pol(&a.g.dout[v[k]], pol_keep));
+#pragma unroll
+            for (int k = 0; k < U; k++) {
+                if (j[k] >= 0) {
+                    const uint32_t sj = s.sid[j[k]];
+                    red_add_pol(Rp<PK>(a.g, sj, v[k]), __ddiv_rn(s.w[j[k]], (double)d[k]), pol_keep);
+                    mark_bit(a.bitmap, (size_t)v[k] * a.g.S + sj);
+                }
+            }
+        }
+        return;
+    }
+#if PPR_PUSH_DYN
+    // warps claim U consecutive 32-edge chunks at a time from a shared counter,
+    // so a warp whose atomics return late does not hold the tile's barrier
+    while (true) {
+        uint32_t cb = 0;
+        if (L == 0) cb = atomicAdd(&s.chunk, (unsigned)U);
+        cb = __shfl_sync(0xffffffffu, cb, 0);
+        if (cb * 32 >= E) break;
+#define PPR_CHUNK(k) (cb + (k))
+#else
     for (uint32_t cb = w; cb * 32 < E; cb += NW * U) {
+#define PPR_CHUNK(k) (cb + NW * (k))
+#endif
         ensure_room(s, c, 32 * U);
         uint32_t v[U];
         int j[U];
 #pragma unroll
         for (int k = 0; k < U; k++) {
-            const uint32_t e = (cb + NW * k) * 32 + L;
+            const uint32_t e = PPR_CHUNK(k) * 32 + L;
             j[k] = -1;
             v[k] = 0;
             if (e < E) {
@@ -413,6 +473,45 @@ __device__ __forceinline__ void clear_frontier_bits(Ctx& c, const PushArgs& a, c
     }
 }
 
+// ---------------------------------------------------------------- bitmap-scan frontier
+//
+// After the round's reductions are complete (grid barrier), every marked
+// (vertex, source) bit is tested once: it joins the next frontier iff its
+// residual meets pushCond.  Words are scanned warp-wide (lane = word), the
+// hits are compacted with ballot/popc into the warp's queue slice, and the
+// words are cleared.  Every vertex whose residual changed this round was
+// marked, and every other residual is unchanged and fails pushCond, so the
+// emitted frontier is exactly {(s,v) : pushCond(R_s(v))} (Alg 3 line 1,
+// restricted to the vertices the round touched) and is sorted by vertex
+// within each warp's word range.
+template <bool POS, bool PK>
+__device__ __forceinline__ void scan_bitmap(Smem& s, Ctx& c, const PushArgs& a) {
+    const double eps = a.g.eps;
+    const uint64_t nbits = (uint64_t)a.g.S * a.g.n;
+    const uint64_t nwords = (nbits + 31) / 32;
+    const uint64_t gw = (uint64_t)blockIdx.x * NW + warp(), nw = (uint64_t)gridDim.x * NW;
+    for (uint64_t w0 = gw * 32; w0 < nwords; w0 += nw * 32) {
+        const uint64_t wi = w0 + lane();
+        uint32_t word = wi < nwords ? __ldcg(&a.bitmap[wi]) : 0u;
+        if (word) __stcg(&a.bitmap[wi], 0u);
+        // lanes drain their words bit by bit; the warp advances while any lane has bits
+        while (__any_sync(0xffffffffu, word != 0)) {
+            bool enq = false;
+            unsigned long long ent = 0;
+            if (word) {
+                const int b = __ffs(word) - 1;
+                word &= word - 1;
+                const uint64_t bit = wi * 32 + b;
+                const uint32_t v = (uint32_t)(bit / a.g.S), sidx = (uint32_t)(bit % a.g.S);
+                enq = push_cond<POS>(__ldcg(Rp<PK>(a.g, sidx, v)), eps);
+                ent = ((unsigned long long)sidx << 32) | v;
+            }
+            ensure_room(s, c, 32);
+            warp_enqueue(s, c, enq, ent);
+        }
+    }
+}
+
 // ---------------------------------------------------------------- seeding
 
 template <bool POS, bool PK>
@@ -493,6 +592,10 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
         const unsigned long long t0 = a.trace ? global_ns() : 0;
         if (MODE == M_OPT) {
             propagate_all<POS, K_OPT, PK>(s, c, a, Fin, C, tc);
+        } else if (MODE == M_SCAN) {
+            propagate_all<POS, K_SCAN, PK>(s, c, a, Fin, C, tc);
+            grid_sync(ctl);  // every reduction of the round has landed
+            scan_bitmap<POS, PK>(s, c, a);
         } else if (MODE == M_VAN || MODE == M_DUP) {
             session_snapshot<PK>(c, a, Fin, C, MODE == M_VAN);
             grid_sync(ctl);
@@ -762,6 +865,7 @@ cudaError_t launch_layout(int mode, const PushArgs& a, int num_sms, cudaStream_t
         case M_DUP: return launch_mode<M_DUP, PK>(a, num_sms, st);
         case M_VAN: return launch_mode<M_VAN, PK>(a, num_sms, st);
         case M_ASYNC: return launch_async<PK>(a, num_sms, st);
+        case M_SCAN: return launch_mode<M_SCAN, PK>(a, num_sms, st);
         default: return cudaErrorInvalidValue;
     }
 }

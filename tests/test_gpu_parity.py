@@ -19,7 +19,7 @@ from tests import golden_figs as G
 
 pytestmark = pytest.mark.gpu
 
-MODES = ["opt", "eager", "dupdetect", "vanilla", "async"]
+MODES = ["opt", "eager", "dupdetect", "vanilla", "async", "scan"]
 
 
 def _fig_gpu(mode="vanilla", max_iters=0):

@@ -78,6 +78,8 @@ struct ppr_ctx {
     int shifts[8] = {0};
     int npasses = 0;
     cudaEvent_t ev[5] = {nullptr, nullptr, nullptr, nullptr, nullptr};
+    cudaStream_t st2 = nullptr;  // restore branch of a batch (fork/join with st)
+    cudaEvent_t ev_fork = nullptr, ev_valid = nullptr, ev_join = nullptr;
     std::string err;
     bool poisoned = false;
     uint64_t dev_bytes = 0;
@@ -161,6 +163,7 @@ void free_batch(ppr_ctx* h) {
         dfree(h, b.ou[i], h->bcap);
     }
     dfree(h, b.hist, rs_hist_entries(h->bcap));
+    dfree(h, b.hist2, rs_hist_entries(h->bcap));
     dfree(h, b.rnv, h->bcap);
     dfree(h, b.rnu, h->bcap);
     dfree(h, b.vheads, h->bcap);
@@ -187,7 +190,8 @@ ppr_status ensure_batch(ppr_ctx* h, uint64_t nupd, uint64_t N) {
         ok = ok && dalloc(h, &b.kv[i], cap) == cudaSuccess && dalloc(h, &b.ku[i], cap) == cudaSuccess &&
              dalloc(h, &b.ov[i], cap) == cudaSuccess && dalloc(h, &b.ou[i], cap) == cudaSuccess;
     }
-    ok = ok && dalloc(h, &b.hist, rs_hist_entries(cap)) == cudaSuccess;
+    ok = ok && dalloc(h, &b.hist, rs_hist_entries(cap)) == cudaSuccess &&
+         dalloc(h, &b.hist2, rs_hist_entries(cap)) == cudaSuccess;
     ok = ok && dalloc(h, &b.rnv, cap) == cudaSuccess && dalloc(h, &b.rnu, cap) == cudaSuccess;
     ok = ok && dalloc(h, &b.vheads, cap) == cudaSuccess && dalloc(h, &b.uheads, cap) == cudaSuccess;
     ok = ok && dalloc(h, &b.claim, cap) == cudaSuccess && dalloc(h, &b.delpos, cap) == cudaSuccess;
@@ -364,6 +368,9 @@ void destroy_all(ppr_ctx* h) {
     h->h_ctl = nullptr;
     for (auto& e : h->ev)
         if (e) cudaEventDestroy(e), e = nullptr;
+    for (cudaEvent_t* e : {&h->ev_fork, &h->ev_valid, &h->ev_join})
+        if (*e) cudaEventDestroy(*e), *e = nullptr;
+    if (h->st2) cudaStreamSynchronize(h->st2), cudaStreamDestroy(h->st2), h->st2 = nullptr;
     dfree(h, h->d_trace, 4ull * h->trace_cap + 8);
     dfree(h, h->d_ring, h->ring_cap);
     if (h->own_stream && h->st) cudaStreamDestroy(h->st);
@@ -472,6 +479,10 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         h->own_stream = true;
     }
     for (auto& ev : h->ev) cudaEventCreate(&ev);
+    cudaStreamCreateWithFlags(&h->st2, cudaStreamNonBlocking);
+    cudaEventCreateWithFlags(&h->ev_fork, cudaEventDisableTiming);
+    cudaEventCreateWithFlags(&h->ev_valid, cudaEventDisableTiming);
+    cudaEventCreateWithFlags(&h->ev_join, cudaEventDisableTiming);
     h->npasses = key_shifts(ceil_log2(h->n), h->shifts);
     if (getenv("PPR_TRACE") && atoi(getenv("PPR_TRACE")) > 0) {
         h->trace_cap = 4096;
@@ -719,25 +730,34 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     launch_ctl_reset(h->d_ctl, st, &launches);
     launch_batch_keys(is, id, n_ins, ds, dd, n_del, h->undirected, h->n, b, 0, h->d_ctl, st,
                       &launches);
-    // two sorts of the same batch: (v,u) for the store, (u,v) for the restore
+    // Fork: the store chain (sort by (v,u), validate, apply/rebuild) stays on
+    // st; the restore chain (sort by (u,v), heads, restore) runs on st2.  The
+    // restore waits for validation so that an invalid batch mutates nothing.
+    cudaEventRecord(h->ev_fork, st);
+    cudaStreamWaitEvent(h->st2, h->ev_fork, 0);
+    cudaStream_t s2 = h->st2;
     int wv = radix_sort_pairs(b.kv[0], b.ov[0], b.kv[1], b.ov[1], N, h->shifts, h->npasses,
                               b.hist, st, &launches);
     int wu = radix_sort_pairs(b.ku[0], b.ou[0], b.ku[1], b.ou[1], N, h->shifts, h->npasses,
-                              b.hist, st, &launches);
+                              b.hist2, s2, &launches);
     const uint64_t* kv = b.kv[wv];
     const uint64_t* ku = b.ku[wu];
     cudaMemsetAsync(b.claim, 0, sizeof(uint32_t) * N, st);
     launch_heads(kv, b.ov[wv], N, b.rnv, b.vheads, &h->d_ctl->st.n_vheads, st, &launches);
-    launch_heads(ku, b.ou[wu], N, b.rnu, b.uheads, &h->d_ctl->st.n_uheads, st, &launches);
+    launch_heads(ku, b.ou[wu], N, b.rnu, b.uheads, &h->d_ctl->st.n_uheads, s2, &launches);
     // a1: graph store
     launch_store_validate(dg, kv, N, b, h->vb, h->d_ctl, h->force_rebuild ? 1 : 0, st, &launches);
+    cudaEventRecord(h->ev_valid, st);
     launch_store_apply(dg, kv, N, b, h->d_ctl, st, &launches);
     StoreParams sp{h->slack, h->min_cap, h->pool_cap[h->active ^ 1u]};
     launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches);
     launch_seg_cleanup(kv, N, b, h->vb, h->d_ctl, st, &launches);
     record(h, 1);
-    // a2: restore
-    launch_restore(dg, ku, N, b, h->vb, h->d_ctl, st, &launches);
+    // a2: restore (after validation)
+    cudaStreamWaitEvent(s2, h->ev_valid, 0);
+    launch_restore(dg, ku, N, b, h->vb, h->d_ctl, s2, &launches);
+    cudaEventRecord(h->ev_join, s2);
+    cudaStreamWaitEvent(st, h->ev_join, 0);  // join
     record(h, 2);
     // a3-a6: push
     if (h->push_enabled) {

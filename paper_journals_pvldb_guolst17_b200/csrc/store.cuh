@@ -16,7 +16,8 @@ struct BatchBufs {
     uint32_t* ov[2];   // op code (0: delete, 1: no-op, 2: insert)
     uint64_t* ku[2];   // keys (u << 32 | v), sorted for the restore
     uint32_t* ou[2];
-    uint32_t* hist;    // radix-sort scratch
+    uint32_t* hist;    // radix-sort scratch (store order)
+    uint32_t* hist2;   // radix-sort scratch (restore order, sorted concurrently)
     int32_t* rnv;      // net multiplicity change at each run head (v-sorted)
     int32_t* rnu;      // same, u-sorted
     uint32_t* vheads;  // v-segment heads

@@ -142,8 +142,8 @@ def make_stream(name, seed=42, **over):
     cfg.update(over)
     src, dst = rmat_stream(cfg["n"], cfg["m"], seed=seed, abc=cfg["abc"],
                            undirected=cfg["undirected"])
-    if cfg["window"] is None:  # resident window: all but the slides' insertions
-        w0 = cfg["m"] - (cfg["slides"] + 5) * cfg["ins"]
+    if cfg["window"] is None:  # resident window: all but the insertions of 2*slides + 5 slides
+        w0 = cfg["m"] - (2 * cfg["slides"] + 5) * cfg["ins"]
     else:
         w0 = int(round(cfg["window"] * cfg["m"]))
     st = Stream(cfg["n"], src, dst, w0, cfg["ins"], cfg["dele"], cfg["undirected"])

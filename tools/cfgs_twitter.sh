@@ -1,0 +1,1 @@
+run twitter --workload twitter --steps 10 --warmup 3

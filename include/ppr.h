@@ -96,6 +96,9 @@ typedef struct {
     int mode;            /* PPR_MODE_* (default PPR_MODE_OPT) */
     double slack;        /* slab slack fraction (default 0.25) */
     uint32_t min_cap;    /* minimum slab capacity (default 4) */
+    int relabel;         /* 1 (default): vertices are renumbered internally by G0 out-degree
+                            (descending) so the most-pushed-to residuals share cache lines;
+                            every id at the boundary stays external.  0: identity. */
 } ppr_opts;
 
 /* Per-call statistics (filled by ppr_create, ppr_apply_batch, ppr_push). */

@@ -63,7 +63,9 @@ struct ppr_ctx {
     uint32_t* d_pool[2] = {nullptr, nullptr};
     double* d_P = nullptr;
     double* d_R = nullptr;
-    uint32_t* d_sources = nullptr;
+    uint32_t* d_sources = nullptr;  // internal ids
+    uint32_t* d_perm = nullptr;     // external -> internal vertex id (degree order), or null
+    uint32_t* d_inv = nullptr;      // internal -> external
     unsigned long long* d_F[2] = {nullptr, nullptr};
     double* d_W = nullptr;
     uint32_t* d_bitmap = nullptr;
@@ -353,6 +355,8 @@ void destroy_all(ppr_ctx* h) {
     dfree(h, h->d_P, (uint64_t)h->S * h->n);
     dfree(h, h->d_R, (uint64_t)h->S * h->n);
     dfree(h, h->d_sources, h->S);
+    dfree(h, h->d_perm, h->n);
+    dfree(h, h->d_inv, h->n);
     dfree(h, h->d_F[0], (uint64_t)h->S * h->n);
     dfree(h, h->d_F[1], (uint64_t)h->S * h->n);
     dfree(h, h->d_W, (uint64_t)h->S * h->n);
@@ -445,6 +449,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     o.mode = PPR_MODE_OPT;
     o.slack = 0.25;
     o.min_cap = 4;
+    o.relabel = 1;
     if (opts) o = *opts;
     if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_EAGER_SCAN || !(o.slack >= 0.0) ||
         o.min_cap == 0)
@@ -573,6 +578,34 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         cudaMemcpyAsync(d_src, g->src, sizeof(uint32_t) * g->m, cudaMemcpyHostToDevice, st);
         cudaMemcpyAsync(d_dst, g->dst, sizeof(uint32_t) * g->m, cudaMemcpyHostToDevice, st);
     }
+    if (o.relabel) {  // degree-ordered internal ids
+        uint64_t *k0 = nullptr, *k1 = nullptr;
+        uint32_t *v0 = nullptr, *v1 = nullptr, *hist = nullptr;
+        bool okr = dalloc(h, &h->d_perm, h->n) == cudaSuccess && dalloc(h, &h->d_inv, h->n) == cudaSuccess &&
+                   dalloc(h, &k0, h->n) == cudaSuccess && dalloc(h, &k1, h->n) == cudaSuccess &&
+                   dalloc(h, &v0, h->n) == cudaSuccess && dalloc(h, &v1, h->n) == cudaSuccess &&
+                   dalloc(h, &hist, rs_hist_entries(h->n)) == cudaSuccess;
+        if (okr) {
+            launch_relabel(d_src, d_dst, g->m, h->undirected, h->n, h->vb.newcap, k0, v0, k1, v1, hist,
+                           h->d_perm, h->d_inv, st, &launches);
+            launch_map_ids(d_src, g->m, h->d_perm, st, &launches);
+            launch_map_ids(d_dst, g->m, h->d_perm, st, &launches);
+            launch_map_ids(h->d_sources, h->S, h->d_perm, st, &launches);
+            cudaStreamSynchronize(st);
+        }
+        dfree(h, k0, h->n);
+        dfree(h, k1, h->n);
+        dfree(h, v0, h->n);
+        dfree(h, v1, h->n);
+        dfree(h, hist, rs_hist_entries(h->n));
+        if (!okr) {
+            dfree(h, d_src, g->m);
+            dfree(h, d_dst, g->m);
+            destroy_all(h);
+            delete h;
+            return PPR_ENOMEM;
+        }
+    }
     DevGraph dg = graph_of(h);
     launch_build_count(d_src, d_dst, g->m, h->undirected, dg, h->n, st, &launches);
     launch_caps_from_len(dg, h->vb, h->slack, h->min_cap, st, &launches);
@@ -617,7 +650,10 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     record(h, 2);
     // static PPR: push from the sources (P = 0, R = e_s)
     std::vector<unsigned long long> seeds(h->S);
-    for (uint32_t i = 0; i < h->S; i++) seeds[i] = ((unsigned long long)i << 32) | sources[i];
+    std::vector<uint32_t> isrc(h->S);  // internal ids of the sources
+    cudaMemcpyAsync(isrc.data(), h->d_sources, sizeof(uint32_t) * h->S, cudaMemcpyDeviceToHost, st);
+    cudaStreamSynchronize(st);
+    for (uint32_t i = 0; i < h->S; i++) seeds[i] = ((unsigned long long)i << 32) | isrc[i];
     unsigned long long* d_seeds = nullptr;
     if (dalloc(h, &d_seeds, h->S) != cudaSuccess) {
         dfree(h, d_src, g->m);
@@ -728,7 +764,7 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     DevGraph dg = graph_of(h);
     BatchBufs& b = h->bb;
     launch_ctl_reset(h->d_ctl, st, &launches);
-    launch_batch_keys(is, id, n_ins, ds, dd, n_del, h->undirected, h->n, b, 0, h->d_ctl, st,
+    launch_batch_keys(is, id, n_ins, ds, dd, n_del, h->undirected, h->n, b, 0, h->d_ctl, h->d_perm, st,
                       &launches);
     // Fork: the store chain (sort by (v,u), validate, apply/rebuild) stays on
     // st; the restore chain (sort by (u,v), heads, restore) runs on st2.  The
@@ -806,7 +842,7 @@ ppr_status ppr_reset(ppr_ctx* h) {
     uint32_t launches = 0;
     const uint64_t Sn = (uint64_t)h->S * h->n;
     if (h->d_rec) {
-        launch_gather_rec(graph_of(h), nullptr, nullptr, nullptr, 1, h->st, &launches);
+        launch_gather_rec(graph_of(h), nullptr, nullptr, nullptr, 1, nullptr, h->st, &launches);
     } else {
         cudaMemsetAsync(h->d_P, 0, sizeof(double) * Sn, h->st);
         cudaMemsetAsync(h->d_R, 0, sizeof(double) * Sn, h->st);
@@ -833,7 +869,7 @@ ppr_status ppr_query(ppr_ctx* h, uint32_t source_idx, double* P_out, double* R_o
         uint32_t launches = 0;
         double* dP = host ? (P_out ? tmp : nullptr) : P_out;
         double* dR = host ? (R_out ? tmp + h->n : nullptr) : R_out;
-        launch_gather_rec(graph_of(h), dP, dR, nullptr, 0, h->st, &launches);
+        launch_gather_rec(graph_of(h), dP, dR, nullptr, 0, h->d_perm, h->st, &launches);
         if (host && P_out) e = cudaMemcpyAsync(P_out, tmp, sizeof(double) * h->n, k, h->st);
         if (host && e == cudaSuccess && R_out)
             e = cudaMemcpyAsync(R_out, tmp + h->n, sizeof(double) * h->n, k, h->st);
@@ -842,7 +878,7 @@ ppr_status ppr_query(ppr_ctx* h, uint32_t source_idx, double* P_out, double* R_o
         if (e != cudaSuccess) return cuda_fail(h, e, "ppr_query");
         return PPR_OK;
     }
-    if (h->S > 1) {  // vertex-major [n][S]: gather the column through a device buffer
+    if (h->S > 1 || h->d_perm) {  // vertex-major [n][S] / internal ids: gather through a device buffer
         double* tmp = nullptr;
         const bool host = mem == PPR_MEM_HOST;
         if (host && dalloc(h, &tmp, h->n) != cudaSuccess) return PPR_ENOMEM;
@@ -851,7 +887,8 @@ ppr_status ppr_query(ppr_ctx* h, uint32_t source_idx, double* P_out, double* R_o
         double* outs[2] = {P_out, R_out};
         for (int q = 0; q < 2 && e == cudaSuccess; q++) {
             if (!outs[q]) continue;
-            launch_gather_col(srcs[q], h->S, source_idx, h->n, host ? tmp : outs[q], h->st, &launches);
+            launch_gather_col(srcs[q], h->S, source_idx, h->n, host ? tmp : outs[q], h->d_perm, h->st,
+                              &launches);
             if (host) e = cudaMemcpyAsync(outs[q], tmp, sizeof(double) * h->n, k, h->st);
             if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
         }
@@ -874,7 +911,18 @@ ppr_status ppr_export_dout(ppr_ctx* h, uint32_t* dout_out) {
         uint32_t* tmp = nullptr;
         uint32_t launches = 0;
         if (dalloc(h, &tmp, h->n) != cudaSuccess) return PPR_ENOMEM;
-        launch_gather_rec(graph_of(h), nullptr, nullptr, tmp, 0, h->st, &launches);
+        launch_gather_rec(graph_of(h), nullptr, nullptr, tmp, 0, h->d_perm, h->st, &launches);
+        e = cudaMemcpyAsync(dout_out, tmp, sizeof(uint32_t) * h->n, cudaMemcpyDeviceToHost, h->st);
+        if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
+        dfree(h, tmp, h->n);
+        if (e != cudaSuccess) return cuda_fail(h, e, "ppr_export_dout");
+        return PPR_OK;
+    }
+    if (h->d_perm) {
+        uint32_t* tmp = nullptr;
+        uint32_t launches = 0;
+        if (dalloc(h, &tmp, h->n) != cudaSuccess) return PPR_ENOMEM;
+        launch_gather_u32(h->d_dout, h->d_perm, h->n, tmp, h->st, &launches);
         e = cudaMemcpyAsync(dout_out, tmp, sizeof(uint32_t) * h->n, cudaMemcpyDeviceToHost, h->st);
         if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
         dfree(h, tmp, h->n);
@@ -914,7 +962,7 @@ ppr_status ppr_export_edges(ppr_ctx* h, uint32_t* src_out, uint32_t* dst_out, ui
         DevGraph dg = graph_of(h);
         launch_len_to_u32(dg, lens, st, &launches);
         exclusive_scan_u32(lens, off, h->n, h->vb.part, &h->d_ctl->st.pool_top, st, &launches);
-        launch_export(dg, (int)h->active, off, k[0], st, &launches);
+        launch_export(dg, (int)h->active, off, k[0], h->d_inv, st, &launches);
         cudaMemsetAsync(v[0], 0, sizeof(uint32_t) * m, st);
         int w = radix_sort_pairs(k[0], v[0], k[1], v[1], m, h->shifts, h->npasses, hist, st,
                                  &launches);

@@ -102,7 +102,8 @@ __global__ void k_batch_keys(const uint32_t* __restrict__ is, const uint32_t* __
                              uint64_t n_ins, const uint32_t* __restrict__ ds,
                              const uint32_t* __restrict__ dd, uint64_t n_del, int undirected,
                              uint32_t n, uint64_t* __restrict__ kv, uint32_t* __restrict__ ov,
-                             uint64_t* __restrict__ ku, uint32_t* __restrict__ ou, DevCtl* ctl) {
+                             uint64_t* __restrict__ ku, uint32_t* __restrict__ ou, DevCtl* ctl,
+                             const uint32_t* __restrict__ perm) {
     const uint64_t tot = n_ins + n_del;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < tot;
          i += (uint64_t)gridDim.x * blockDim.x) {
@@ -114,6 +115,9 @@ __global__ void k_batch_keys(const uint32_t* __restrict__ is, const uint32_t* __
             set_err(ctl, KERR_RANGE);
             u = v = 0;
             op = 1u;
+        } else if (perm) {  // internal (degree-ordered) vertex ids
+            u = perm[u];
+            v = perm[v];
         }
         if (!undirected) {
             kv[i] = ((uint64_t)v << 32) | u;
@@ -557,21 +561,73 @@ __global__ void k_len_to_u32(DevGraph g, uint32_t* __restrict__ out) {
 
 template <bool PK>
 __global__ void k_export(DevGraph g, int active, const unsigned long long* __restrict__ off,
-                         uint64_t* __restrict__ keys) {
+                         uint64_t* __restrict__ keys, const uint32_t* __restrict__ inv) {
     const uint32_t* pool = g.pool[active];
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x) {
         const Slab sl = get_slab<PK>(g, v);
-        for (uint32_t j = 0; j < sl.len; j++) keys[off[v] + j] = (v << 32) | pool[sl.off + j];
+        const uint64_t vo = inv ? inv[v] : v;  // external id
+        for (uint32_t j = 0; j < sl.len; j++) {
+            const uint32_t x = pool[sl.off + j];
+            keys[off[v] + j] = (vo << 32) | (inv ? inv[x] : x);
+        }
     }
+}
+
+// ---------------------------------------------------------------- degree-ordered relabelling
+// Vertices are renumbered by G0 out-degree (descending, ties by id) so that
+// the heaviest receivers of pushes (a vertex is pushed to once per frontier
+// out-neighbour) share residual / d_out cache lines.  perm: external ->
+// internal id, inv: internal -> external.
+
+__global__ void k_count_out(const uint32_t* __restrict__ src, const uint32_t* __restrict__ dst,
+                            uint64_t m, int undirected, uint32_t* __restrict__ deg) {
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
+         i += (uint64_t)gridDim.x * blockDim.x) {
+        atomicAdd(&deg[src[i]], 1u);
+        if (undirected && src[i] != dst[i]) atomicAdd(&deg[dst[i]], 1u);
+    }
+}
+
+__global__ void k_degree_keys(const uint32_t* __restrict__ deg, uint32_t n, uint64_t* __restrict__ keys,
+                              uint32_t* __restrict__ vals) {
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
+         v += (uint64_t)gridDim.x * blockDim.x) {
+        keys[v] = ((uint64_t)(0xFFFFFFFFu - deg[v]) << 32) | v;
+        vals[v] = 0;
+    }
+}
+
+__global__ void k_perm_from_sorted(const uint64_t* __restrict__ keys, uint32_t n,
+                                   uint32_t* __restrict__ perm, uint32_t* __restrict__ inv) {
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+         i += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t v = (uint32_t)keys[i];
+        inv[i] = v;
+        perm[v] = (uint32_t)i;
+    }
+}
+
+__global__ void k_map_ids(uint32_t* __restrict__ a, uint64_t m, const uint32_t* __restrict__ perm) {
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
+         i += (uint64_t)gridDim.x * blockDim.x)
+        a[i] = perm[a[i]];
+}
+
+__global__ void k_gather_u32(const uint32_t* __restrict__ src, const uint32_t* __restrict__ perm,
+                             uint32_t n, uint32_t* __restrict__ dst) {
+    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
+         v += (uint64_t)gridDim.x * blockDim.x)
+        dst[v] = src[perm ? perm[v] : v];
 }
 
 // packed layout: P, R, d_out out of the records (query / export / reset)
 __global__ void k_gather_rec(DevGraph g, double* __restrict__ P, double* __restrict__ R,
-                             uint32_t* __restrict__ dout, int zero_pr) {
+                             uint32_t* __restrict__ dout, int zero_pr,
+                             const uint32_t* __restrict__ perm) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x) {
-        VRec* rc = &g.rec[v];
+        VRec* rc = &g.rec[perm ? perm[v] : v];
         if (P) P[v] = rc->p;
         if (R) R[v] = rc->r;
         if (dout) dout[v] = rc->dout;
@@ -581,10 +637,10 @@ __global__ void k_gather_rec(DevGraph g, double* __restrict__ P, double* __restr
 
 // arrays layout, S > 1: column `sidx` of a vertex-major [n][S] array
 __global__ void k_gather_col(const double* __restrict__ src, uint32_t S, uint32_t sidx, uint32_t n,
-                             double* __restrict__ dst) {
+                             double* __restrict__ dst, const uint32_t* __restrict__ perm) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
          v += (uint64_t)gridDim.x * blockDim.x)
-        dst[v] = src[v * S + sidx];
+        dst[v] = src[(uint64_t)(perm ? perm[v] : v) * S + sidx];
 }
 
 // the kernel instance for the handle's layout
@@ -606,11 +662,11 @@ void launch_ctl_reset(DevCtl* ctl, cudaStream_t st, uint32_t* launches) {
 
 void launch_batch_keys(const uint32_t* is, const uint32_t* id, uint64_t n_ins, const uint32_t* ds,
                        const uint32_t* dd, uint64_t n_del, int undirected, uint32_t n,
-                       const BatchBufs& b, int slot, DevCtl* ctl, cudaStream_t st,
-                       uint32_t* launches) {
+                       const BatchBufs& b, int slot, DevCtl* ctl, const uint32_t* perm,
+                       cudaStream_t st, uint32_t* launches) {
     k_batch_keys<<<grid_for(n_ins + n_del, 256), 256, 0, st>>>(
         is, id, n_ins, ds, dd, n_del, undirected, n, b.kv[slot], b.ov[slot], b.ku[slot],
-        b.ou[slot], ctl);
+        b.ou[slot], ctl, perm);
     ++*launches;
 }
 
@@ -699,20 +755,49 @@ void launch_init_state(const DevGraph& g, cudaStream_t st, uint32_t* launches) {
 }
 
 void launch_export(const DevGraph& g, int active, const unsigned long long* off, uint64_t* keys,
-                   cudaStream_t st, uint32_t* launches) {
-    LAUNCH_PK(k_export)<<<grid_for(g.n, 256), 256, 0, st>>>(g, active, off, keys);
+                   const uint32_t* inv, cudaStream_t st, uint32_t* launches) {
+    LAUNCH_PK(k_export)<<<grid_for(g.n, 256), 256, 0, st>>>(g, active, off, keys, inv);
     ++*launches;
 }
 
 void launch_gather_rec(const DevGraph& g, double* P, double* R, uint32_t* dout, int zero_pr,
-                       cudaStream_t st, uint32_t* launches) {
-    k_gather_rec<<<grid_for(g.n, 256), 256, 0, st>>>(g, P, R, dout, zero_pr);
+                       const uint32_t* perm, cudaStream_t st, uint32_t* launches) {
+    k_gather_rec<<<grid_for(g.n, 256), 256, 0, st>>>(g, P, R, dout, zero_pr, perm);
     ++*launches;
 }
 
 void launch_gather_col(const double* src, uint32_t S, uint32_t sidx, uint32_t n, double* dst,
+                       const uint32_t* perm, cudaStream_t st, uint32_t* launches) {
+    k_gather_col<<<grid_for(n, 256), 256, 0, st>>>(src, S, sidx, n, dst, perm);
+    ++*launches;
+}
+
+void launch_relabel(const uint32_t* src, const uint32_t* dst, uint64_t m, int undirected, uint32_t n,
+                    uint32_t* deg, uint64_t* k0, uint32_t* v0, uint64_t* k1, uint32_t* v1,
+                    uint32_t* hist, uint32_t* perm, uint32_t* inv, cudaStream_t st,
+                    uint32_t* launches) {
+    cudaMemsetAsync(deg, 0, sizeof(uint32_t) * n, st);
+    k_count_out<<<grid_for(m, 256), 256, 0, st>>>(src, dst, m, undirected, deg);
+    k_degree_keys<<<grid_for(n, 256), 256, 0, st>>>(deg, n, k0, v0);
+    int shifts[8], np = 0, lg = 0;
+    while ((1ull << lg) < n) lg++;
+    for (int s = 0; s < lg; s += 8) shifts[np++] = s;
+    for (int s = 32; s < 64; s += 8) shifts[np++] = s;
+    const int w = radix_sort_pairs(k0, v0, k1, v1, n, shifts, np, hist, st, launches);
+    k_perm_from_sorted<<<grid_for(n, 256), 256, 0, st>>>(w ? k1 : k0, n, perm, inv);
+    *launches += 3;
+}
+
+void launch_map_ids(uint32_t* a, uint64_t m, const uint32_t* perm, cudaStream_t st,
+                    uint32_t* launches) {
+    if (!m) return;
+    k_map_ids<<<grid_for(m, 256), 256, 0, st>>>(a, m, perm);
+    ++*launches;
+}
+
+void launch_gather_u32(const uint32_t* src, const uint32_t* perm, uint32_t n, uint32_t* dst,
                        cudaStream_t st, uint32_t* launches) {
-    k_gather_col<<<grid_for(n, 256), 256, 0, st>>>(src, S, sidx, n, dst);
+    k_gather_u32<<<grid_for(n, 256), 256, 0, st>>>(src, perm, n, dst);
     ++*launches;
 }
 

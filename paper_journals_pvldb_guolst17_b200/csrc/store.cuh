@@ -50,8 +50,8 @@ void launch_ctl_reset(DevCtl* ctl, cudaStream_t st, uint32_t* launches);
 // a0: keys of both sort orders + id range check
 void launch_batch_keys(const uint32_t* is, const uint32_t* id, uint64_t n_ins, const uint32_t* ds,
                        const uint32_t* dd, uint64_t n_del, int undirected, uint32_t n,
-                       const BatchBufs& b, int slot, DevCtl* ctl, cudaStream_t st,
-                       uint32_t* launches);
+                       const BatchBufs& b, int slot, DevCtl* ctl, const uint32_t* perm,
+                       cudaStream_t st, uint32_t* launches);
 
 // run nets + segment heads of a sorted key array
 void launch_heads(const uint64_t* keys, const uint32_t* ops, uint64_t N, int32_t* run_net,
@@ -87,13 +87,22 @@ void launch_init_state(const DevGraph& g, cudaStream_t st, uint32_t* launches);
 
 // export: (v << 32 | u) keys of every arc into keys[0..m)
 void launch_export(const DevGraph& g, int active, const unsigned long long* off, uint64_t* keys,
-                   cudaStream_t st, uint32_t* launches);
+                   const uint32_t* inv, cudaStream_t st, uint32_t* launches);
+// degree-ordered relabelling: perm (external -> internal), inv (internal -> external)
+void launch_relabel(const uint32_t* src, const uint32_t* dst, uint64_t m, int undirected, uint32_t n,
+                    uint32_t* deg, uint64_t* k0, uint32_t* v0, uint64_t* k1, uint32_t* v1,
+                    uint32_t* hist, uint32_t* perm, uint32_t* inv, cudaStream_t st,
+                    uint32_t* launches);
+void launch_map_ids(uint32_t* a, uint64_t m, const uint32_t* perm, cudaStream_t st,
+                    uint32_t* launches);
+void launch_gather_u32(const uint32_t* src, const uint32_t* perm, uint32_t n, uint32_t* dst,
+                       cudaStream_t st, uint32_t* launches);
 void launch_len_to_u32(const DevGraph& g, uint32_t* out, cudaStream_t st, uint32_t* launches);
 // arrays layout: dst[v] = src[v * S + sidx]
 void launch_gather_col(const double* src, uint32_t S, uint32_t sidx, uint32_t n, double* dst,
-                       cudaStream_t st, uint32_t* launches);
+                       const uint32_t* perm, cudaStream_t st, uint32_t* launches);
 // packed layout: copy P / R / d_out (any may be null) out of the records; zero_pr clears P and R
 void launch_gather_rec(const DevGraph& g, double* P, double* R, uint32_t* dout, int zero_pr,
-                       cudaStream_t st, uint32_t* launches);
+                       const uint32_t* perm, cudaStream_t st, uint32_t* launches);
 
 }  // namespace ppr

@@ -59,7 +59,8 @@ def parse():
     p.add_argument("--ref-budget-s", type=float, default=150.0)
     p.add_argument("--no-flush", action="store_true")
     p.add_argument("--no-e2e", action="store_true")
-    p.add_argument("--no-relabel", action="store_true", help="keep external vertex ids internally")
+    p.add_argument("--relabel", type=int, default=-1,
+                   help="1: degree-ordered internal ids, 0: external ids, -1: by size (default)")
     return p.parse_args()
 
 
@@ -224,7 +225,7 @@ def config_block(args, cfg, eps, S):
             "undirected": cfg["undirected"], "alpha": 0.15, "eps": eps,
             "source_band": f"top-{cfg['band']} out-degree", "sources": S,
             "rmat_abc": list(cfg["abc"]), "mode": args.mode,
-            "internal_ids": "external" if args.no_relabel else "G0 out-degree order",
+            "internal_ids": {1: "G0 out-degree order", 0: "external", -1: "auto (degree order iff R+d_out > 48 MB)"}[args.relabel],
             "l2": ("persisting lines reset + flushed between steps (512 MiB write)"
                    if not args.no_flush else "not flushed")}
 
@@ -306,7 +307,7 @@ def run_ours(args):
     t0 = time.perf_counter()
     h = ppr.Ppr(cfg["n"], win_np[0], win_np[1], my_srcs, alpha=0.15, eps=eps, mode=args.mode,
                 device=local, stream=ctypes_stream(stream), undirected=und,
-                relabel=not args.no_relabel)
+                relabel=args.relabel)
     torch.cuda.synchronize()
     t_create = time.perf_counter() - t0
     create_stats = h.create_stats

@@ -449,7 +449,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     o.mode = PPR_MODE_OPT;
     o.slack = 0.25;
     o.min_cap = 4;
-    o.relabel = 1;
+    o.relabel = -1;
     if (opts) o = *opts;
     if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_EAGER_SCAN || !(o.slack >= 0.0) ||
         o.min_cap == 0)
@@ -578,7 +578,9 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         cudaMemcpyAsync(d_src, g->src, sizeof(uint32_t) * g->m, cudaMemcpyHostToDevice, st);
         cudaMemcpyAsync(d_dst, g->dst, sizeof(uint32_t) * g->m, cudaMemcpyHostToDevice, st);
     }
-    if (o.relabel) {  // degree-ordered internal ids
+    const bool relabel = o.relabel > 0 ||
+                         (o.relabel < 0 && 8.0 * (double)Sn + 4.0 * h->n > 48.0 * 1024 * 1024);
+    if (relabel) {  // degree-ordered internal ids
         uint64_t *k0 = nullptr, *k1 = nullptr;
         uint32_t *v0 = nullptr, *v1 = nullptr, *hist = nullptr;
         bool okr = dalloc(h, &h->d_perm, h->n) == cudaSuccess && dalloc(h, &h->d_inv, h->n) == cudaSuccess &&

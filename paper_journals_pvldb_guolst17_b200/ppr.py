@@ -131,7 +131,7 @@ class Ppr:
     """One PPR handle (one graph, S sources) on one GPU."""
 
     def __init__(self, n, src, dst, sources, alpha=0.15, eps=1e-9, mode="opt", device=0,
-                 stream=None, undirected=False, slack=0.25, min_cap=4, relabel=True):
+                 stream=None, undirected=False, slack=0.25, min_cap=4, relabel=-1):
         lib = load()
         s, sp = _host_u32(src)
         d, dp = _host_u32(dst)
@@ -140,7 +140,7 @@ class Ppr:
         g = Graph(n=int(n), m=len(s), src=ctypes.cast(sp, ctypes.POINTER(ctypes.c_uint32)),
                   dst=ctypes.cast(dp, ctypes.POINTER(ctypes.c_uint32)), undirected=int(undirected))
         o = Opts(device=int(device), cuda_stream=stream, mode=MODES.get(mode, mode),
-                 slack=float(slack), min_cap=int(min_cap), relabel=int(bool(relabel)))
+                 slack=float(slack), min_cap=int(min_cap), relabel=int(relabel))
         h = ctypes.c_void_p()
         st = BatchStats()
         rc = lib.ppr_create(ctypes.byref(g), ctypes.cast(sop, ctypes.POINTER(ctypes.c_uint32)),

@@ -106,13 +106,13 @@ def _check_batch_state(h, o, sidx, s, eps, what):
     return P, Po
 
 
-def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, **over):
+def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, relabel=-1, **over):
     st, cfg = W.make_stream(name, **over)
     eps = eps or cfg["eps"]
     g0s, g0d = st.window()
     srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], sources)
     h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=eps, mode=mode,
-                undirected=False)
+                undirected=False, relabel=relabel)
     o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, eps)
     o.push(oracle.SEQ)
     for i, s in enumerate(srcs):
@@ -134,6 +134,27 @@ def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, **over):
 @pytest.mark.parametrize("mode", MODES)
 def test_tiny_config_all_modes_track_oracle(mode):
     _run_stream("tiny", mode, slides=12)
+
+
+@pytest.mark.parametrize("mode", ["opt", "scan", "vanilla"])
+def test_tiny_config_degree_relabelled(mode):
+    # internal degree-ordered ids: every id at the boundary must stay external
+    _run_stream("tiny", mode, slides=8, relabel=1)
+
+
+def test_tiny_config_multi_source_relabelled():
+    _run_stream("tiny", "opt", slides=4, sources=3, relabel=1)
+
+
+def test_fig2_bit_exact_with_relabelling():
+    h = ppr.Ppr(G.N, G.G0_SRC, G.G0_DST, [G.SOURCE], alpha=G.ALPHA, eps=G.EPS, mode="vanilla",
+                relabel=1)
+    h.apply_batch([0, 3], [1, 0])
+    P, R = h.query()
+    np.testing.assert_array_equal(R, [7 / 128, 5 / 64, 5 / 128, 5 / 128])
+    np.testing.assert_array_equal(P, [37 / 64, 1 / 4, 3 / 16, 11 / 64])
+    d = h.export_dout()
+    np.testing.assert_array_equal(d, [2, 1, 2, 2])
 
 
 def test_tiny_config_full_50_slides_opt():

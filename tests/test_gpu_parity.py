@@ -330,3 +330,46 @@ def test_undirected_stream():
         h.apply_batch(*b)
         o.apply(*b)
         _check_batch_state(h, o, 0, int(srcs[0]), 1e-8, f"undirected slide {t}")
+
+
+# ---------------------------------------------------------------- full BASELINE sizes
+
+def test_lj_full_size_against_oracle():
+    """configs[1] at full size in the bench's launch configuration (Opt mode,
+    degree relabelling on): the static state and two 10^4+10^4 slides, every
+    vertex checked -- arc multiset bit-exact, Eq. 2, termination, L_inf <= 2 eps
+    against the sequential oracle."""
+    st, cfg = W.make_stream("lj")
+    g0s, g0d = st.window()
+    (s,) = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 1)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, [s], alpha=0.15, eps=cfg["eps"], mode="opt")
+    o = oracle.Oracle(cfg["n"], g0s, g0d, [s], 0.15, cfg["eps"])
+    o.push(oracle.SEQ)
+    _check_batch_state(h, o, 0, int(s), cfg["eps"], "lj static")
+    for t in range(2):
+        b = st.next_batch()
+        stats = h.apply_batch(*b)
+        o.apply(*b)
+        assert stats["pushed_edges"] > 10**6  # a real hub-band workload
+        _check_batch_state(h, o, 0, int(s), cfg["eps"], f"lj slide {t}")
+
+
+def test_orkut_full_size_properties():
+    """configs[2] shape at full size (undirected, 50% window, deletion-heavy
+    k = 10^4): termination and Eq. 2 at every vertex, arc count bookkeeping."""
+    st, cfg = W.make_stream("orkut")
+    e0s, e0d = st.src[st.lo:st.hi].copy(), st.dst[st.lo:st.hi].copy()
+    arcs = W.expand_undirected(e0s, e0d)
+    (s,) = W.pick_sources(cfg["n"], arcs[0], arcs[1], cfg["band"], 1)
+    h = ppr.Ppr(cfg["n"], e0s, e0d, [s], alpha=0.15, eps=cfg["eps"], undirected=True)
+    assert h.create_stats["num_arcs"] == len(arcs[0])
+    for t in range(2):
+        i0, i1, d0, d1 = st.hi, st.hi + cfg["ins"], st.lo, st.lo + cfg["dele"]
+        stats = h.apply_batch(st.src[i0:i1], st.dst[i0:i1], st.src[d0:d1], st.dst[d0:d1])
+        st.hi, st.lo = i1, d1
+        assert stats["num_arcs"] == 2 * (st.hi - st.lo)
+    P, R = h.query()
+    assert exact.terminated(R, cfg["eps"])
+    gs, gd = h.export_edges()
+    ok, worst = exact.invariant_ok(cfg["n"], gs, gd, int(s), 0.15, P, R)
+    assert ok, worst

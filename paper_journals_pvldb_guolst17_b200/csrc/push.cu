@@ -165,7 +165,12 @@ __device__ __forceinline__ bool test_and_set(uint32_t* bitmap, unsigned long lon
 }
 
 __device__ __forceinline__ void mark_bit(uint32_t* bitmap, unsigned long long bit) {
-    atomicOr(&bitmap[bit >> 5], 1u << (bit & 31u));  // result unused: RED.OR
+    // Test before set: hub vertices are pushed to many times per round, and an
+    // unconditional RED.OR flood on their few words serialises at the L2 slice.
+    // The test load may be stale (L1, invalidated at every grid barrier); a
+    // stale 0 only costs a redundant RED.OR.
+    const uint32_t m = 1u << (bit & 31u);
+    if (!(bitmap[bit >> 5] & m)) atomicOr(&bitmap[bit >> 5], m);  // result unused: RED.OR
 }
 
 __device__ __forceinline__ void clear_bit(uint32_t* bitmap, unsigned long long bit) {

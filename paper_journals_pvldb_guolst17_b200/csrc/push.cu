@@ -276,7 +276,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     }
     const unsigned long long pol_keep = l2_keep(), pol_stream = l2_stream();
     // 32-edge chunks dealt round-robin to the warps (chunk w + NW*i), U per step
-    if (KIND == K_SCAN) {  // fire-and-forget edge walk: no enqueue decisions here
+    if constexpr (KIND == K_SCAN) {  // fire-and-forget edge walk: no enqueue decisions here
         for (uint32_t cb = w; cb * 32 < E; cb += NW * U) {
             uint32_t v[U], d[U];
             int j[U];
@@ -302,8 +302,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
                 }
             }
         }
-        return;
-    }
+    } else {
 #if PPR_PUSH_DYN
     // warps claim U consecutive 32-edge chunks at a time from a shared counter,
     // so a warp whose atomics return late does not hold the tile's barrier
@@ -392,6 +391,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
         ensure_room(s, c, 32);
         warp_enqueue(s, c, re, ent);
     }
+    }  // not K_SCAN
 }
 
 // Every CTA takes tiles of T entries: its first tile statically, the rest by

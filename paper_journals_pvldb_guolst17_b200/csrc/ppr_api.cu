@@ -33,6 +33,24 @@
 
 using namespace ppr;
 
+// shape of a captured batch graph: replay only while all of it matches
+struct GraphKey {
+    uint64_t n_ins = 0, n_del = 0;
+    bool push = false;
+    int mode = -1;
+    uint32_t max_iters = 0;
+    bool timing = false, force_rebuild = false;
+    uint64_t epoch = 0, cap0 = 0, cap1 = 0;
+    const void* pool0 = nullptr;
+    const void* pool1 = nullptr;
+    bool operator==(const GraphKey& o) const {
+        return n_ins == o.n_ins && n_del == o.n_del && push == o.push && mode == o.mode &&
+               max_iters == o.max_iters && timing == o.timing && force_rebuild == o.force_rebuild &&
+               epoch == o.epoch && cap0 == o.cap0 && cap1 == o.cap1 && pool0 == o.pool0 &&
+               pool1 == o.pool1;
+    }
+};
+
 struct ppr_ctx {
     int device = 0;
     cudaStream_t st = nullptr;
@@ -86,6 +104,11 @@ struct ppr_ctx {
     bool poisoned = false;
     uint64_t dev_bytes = 0;
     std::vector<void*> allocs;
+    bool graphs = true;                     // replay each batch shape as a CUDA graph (PPR_GRAPHS=0: off)
+    cudaGraphExec_t gexec = nullptr;
+    GraphKey gkey{};
+    uint32_t glaunches = 0;
+    uint64_t buf_epoch = 0;                 // bumped whenever batch / pool buffers are reallocated
     unsigned long long* d_ring = nullptr;   // PPR_MODE_ASYNC ring queue (2*S*n slots, EMPTY)
     unsigned long long ring_cap = 0;
     unsigned long long* d_trace = nullptr;  // PPR_TRACE=1: per-round trace of the push
@@ -184,6 +207,7 @@ ppr_status ensure_batch(ppr_ctx* h, uint64_t nupd, uint64_t N) {
     cudaError_t e = cudaStreamSynchronize(h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, "ensure_batch sync");
     free_batch(h);
+    h->buf_epoch++;
     uint64_t cap = std::max<uint64_t>(N + N / 4, 1024);
     uint64_t ucap = std::max<uint64_t>(nupd + nupd / 4, 1024);
     BatchBufs& b = h->bb;
@@ -221,6 +245,7 @@ ppr_status ensure_alt_pool(ppr_ctx* h, uint64_t new_arcs) {
     if (e != cudaSuccess) return cuda_fail(h, e, "ensure_alt_pool sync");
     dfree(h, h->d_pool[alt], h->pool_cap[alt]);
     h->pool_cap[alt] = 0;
+    h->buf_epoch++;
     uint64_t cap = need + need / 4;
     if (dalloc(h, &h->d_pool[alt], cap) != cudaSuccess) {
         set_err(h, "out of device memory for the rebuild pool (%llu entries)",
@@ -323,17 +348,23 @@ ppr_status finish(ppr_ctx* h, const char* where) {
     cudaError_t e = cudaMemcpyAsync(h->h_ctl, &h->d_ctl->st, sizeof(DevStats), cudaMemcpyDeviceToHost, h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, where);
     e = cudaStreamSynchronize(h->st);
-    if (e == cudaSuccess) e = cudaGetLastError();
-    if (e != cudaSuccess) return cuda_fail(h, e, where);
+    if (e != cudaSuccess) return cuda_fail(h, e, (std::string(where) + " (stream)").c_str());
+    e = cudaGetLastError();
+    if (e != cudaSuccess) return cuda_fail(h, e, (std::string(where) + " (last error)").c_str());
     return status_of_kerr(h, h->h_ctl->err);
 }
 
 void record(ppr_ctx* h, int i) {
-    if (h->timing) cudaEventRecord(h->ev[i], h->st);
+    if (h->timing) {
+        cudaError_t e = cudaEventRecord(h->ev[i], h->st);
+        if (e != cudaSuccess && getenv("PPR_DEBUG"))
+            fprintf(stderr, "PPR_DEBUG: event record %d: %s\n", i, cudaGetErrorString(e));
+    }
 }
 
 void destroy_all(ppr_ctx* h) {
     if (h->st) cudaStreamSynchronize(h->st);
+    if (h->gexec) cudaGraphExecDestroy(h->gexec), h->gexec = nullptr;
     free_batch(h);
     dfree(h, h->d_rec, h->n);
     if (h->l2_window && h->st) {  // drop the window from the (possibly caller's) stream
@@ -381,21 +412,91 @@ void destroy_all(ppr_ctx* h) {
     h->st = nullptr;
 }
 
+ppr_status ensure_ring(ppr_ctx* h) {
+    if (h->d_ring) return PPR_OK;
+    const uint64_t cap = 2ull * h->S * h->n + 1024;
+    if (dalloc(h, &h->d_ring, cap) != cudaSuccess) {
+        set_err(h, "out of device memory for the async ring (%llu slots)", (unsigned long long)cap);
+        return PPR_ENOMEM;
+    }
+    h->ring_cap = cap;
+    cudaMemsetAsync(h->d_ring, 0xFF, sizeof(unsigned long long) * cap, h->st);
+    return PPR_OK;
+}
+
 ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
     if (h->mode == PPR_MODE_ASYNC && !h->d_ring) {
-        const uint64_t cap = 2ull * h->S * h->n + 1024;
-        if (dalloc(h, &h->d_ring, cap) != cudaSuccess) {
-            set_err(h, "out of device memory for the async ring (%llu slots)", (unsigned long long)cap);
-            return PPR_ENOMEM;
-        }
-        h->ring_cap = cap;
-        cudaMemsetAsync(h->d_ring, 0xFF, sizeof(unsigned long long) * cap, h->st);
+        ppr_status rs = ensure_ring(h);
+        if (rs != PPR_OK) return rs;
     }
     a.ring = h->d_ring;
     a.ring_cap = h->ring_cap;
     cudaError_t e = launch_push(h->mode, a, h->num_sms, h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, "push launch");
     ++*launches;
+    return PPR_OK;
+}
+
+// The device work of one batch after staging (captured into a CUDA graph and
+// replayed, or launched directly): keys, two sorts on two streams, store,
+// restore, push.
+// PPR_DEBUG=1: report the first launch error of a batch with the step that raised it
+inline void dbg_step(const char* what) {
+    static const bool on = getenv("PPR_DEBUG") && atoi(getenv("PPR_DEBUG")) > 0;
+    if (!on) return;
+    cudaError_t e = cudaPeekAtLastError();
+    if (e != cudaSuccess) fprintf(stderr, "PPR_DEBUG: %s: %s\n", what, cudaGetErrorString(e));
+}
+
+ppr_status enqueue_batch(ppr_ctx* h, const uint32_t* is, const uint32_t* id, uint64_t n_ins,
+                         const uint32_t* ds, const uint32_t* dd, uint64_t n_del, uint64_t N,
+                         uint32_t* launches_out) {
+    cudaStream_t st = h->st;
+    uint32_t launches = 0;
+    DevGraph dg = graph_of(h);
+    BatchBufs& b = h->bb;
+    launch_ctl_reset(h->d_ctl, st, &launches);
+    dbg_step("launch_ctl_reset");
+    launch_batch_keys(is, id, n_ins, ds, dd, n_del, h->undirected, h->n, b, 0, h->d_ctl, h->d_perm, st,
+                      &launches);
+    dbg_step("launch_batch_keys");
+    // Fork: the store chain (sort by (v,u), validate, apply/rebuild) stays on
+    // st; the restore chain (sort by (u,v), heads, restore) runs on st2.  The
+    // restore waits for validation so that an invalid batch mutates nothing.
+    cudaEventRecord(h->ev_fork, st);
+    cudaStreamWaitEvent(h->st2, h->ev_fork, 0);
+    cudaStream_t s2 = h->st2;
+    int wv = radix_sort_pairs(b.kv[0], b.ov[0], b.kv[1], b.ov[1], N, h->shifts, h->npasses,
+                              b.hist, st, &launches);
+    dbg_step("radix_sort_pairs");
+    int wu = radix_sort_pairs(b.ku[0], b.ou[0], b.ku[1], b.ou[1], N, h->shifts, h->npasses,
+                              b.hist2, s2, &launches);
+    dbg_step("radix_sort_pairs");
+    const uint64_t* kv = b.kv[wv];
+    const uint64_t* ku = b.ku[wu];
+    cudaMemsetAsync(b.claim, 0, sizeof(uint32_t) * N, st);
+    launch_heads(kv, b.ov[wv], N, b.rnv, b.vheads, &h->d_ctl->st.n_vheads, st, &launches);
+    dbg_step("launch_heads");
+    launch_heads(ku, b.ou[wu], N, b.rnu, b.uheads, &h->d_ctl->st.n_uheads, s2, &launches);
+    dbg_step("launch_heads");
+    // a1: graph store
+    launch_store_validate(dg, kv, N, b, h->vb, h->d_ctl, h->force_rebuild ? 1 : 0, st, &launches);
+    dbg_step("launch_store_validate");
+    cudaEventRecord(h->ev_valid, st);
+    launch_store_apply(dg, kv, N, b, h->d_ctl, st, &launches);
+    dbg_step("launch_store_apply");
+    StoreParams sp{h->slack, h->min_cap, h->pool_cap[h->active ^ 1u]};
+    launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches);
+    dbg_step("launch_store_rebuild");
+    launch_seg_cleanup(kv, N, b, h->vb, h->d_ctl, st, &launches);
+    dbg_step("launch_seg_cleanup");
+    // a2: restore (after validation)
+    cudaStreamWaitEvent(s2, h->ev_valid, 0);
+    launch_restore(dg, ku, N, b, h->vb, h->d_ctl, s2, &launches);
+    dbg_step("launch_restore");
+    cudaEventRecord(h->ev_join, s2);
+    cudaStreamWaitEvent(st, h->ev_join, 0);  // join
+    *launches_out = launches;
     return PPR_OK;
 }
 
@@ -489,6 +590,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     cudaEventCreateWithFlags(&h->ev_valid, cudaEventDisableTiming);
     cudaEventCreateWithFlags(&h->ev_join, cudaEventDisableTiming);
     h->npasses = key_shifts(ceil_log2(h->n), h->shifts);
+    if (getenv("PPR_GRAPHS") && !strcmp(getenv("PPR_GRAPHS"), "0")) h->graphs = false;
     if (getenv("PPR_TRACE") && atoi(getenv("PPR_TRACE")) > 0) {
         h->trace_cap = 4096;
         dalloc(h, &h->d_trace, 4ull * h->trace_cap + 8);
@@ -748,61 +850,77 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     cudaStream_t st = h->st;
     uint32_t launches = 0;
     record(h, 0);
+    // a0: stage the batch in the handle's buffers (H2D, or D2D when the work is a replayed graph)
+    const bool use_graph = h->graphs && !h->d_trace;
     const uint32_t *is = ins_src, *id = ins_dst, *ds = del_src, *dd = del_dst;
-    if (mem == PPR_MEM_HOST) {
+    if (mem == PPR_MEM_HOST || use_graph) {
+        const cudaMemcpyKind kind = mem == PPR_MEM_HOST ? cudaMemcpyHostToDevice : cudaMemcpyDeviceToDevice;
         if (n_ins) {
-            cudaMemcpyAsync(h->d_in[0], ins_src, 4 * n_ins, cudaMemcpyHostToDevice, st);
-            cudaMemcpyAsync(h->d_in[1], ins_dst, 4 * n_ins, cudaMemcpyHostToDevice, st);
+            cudaMemcpyAsync(h->d_in[0], ins_src, 4 * n_ins, kind, st);
+            cudaMemcpyAsync(h->d_in[1], ins_dst, 4 * n_ins, kind, st);
         }
         if (n_del) {
-            cudaMemcpyAsync(h->d_in[2], del_src, 4 * n_del, cudaMemcpyHostToDevice, st);
-            cudaMemcpyAsync(h->d_in[3], del_dst, 4 * n_del, cudaMemcpyHostToDevice, st);
+            cudaMemcpyAsync(h->d_in[2], del_src, 4 * n_del, kind, st);
+            cudaMemcpyAsync(h->d_in[3], del_dst, 4 * n_del, kind, st);
         }
         is = h->d_in[0];
         id = h->d_in[1];
         ds = h->d_in[2];
         dd = h->d_in[3];
     }
-    DevGraph dg = graph_of(h);
-    BatchBufs& b = h->bb;
-    launch_ctl_reset(h->d_ctl, st, &launches);
-    launch_batch_keys(is, id, n_ins, ds, dd, n_del, h->undirected, h->n, b, 0, h->d_ctl, h->d_perm, st,
-                      &launches);
-    // Fork: the store chain (sort by (v,u), validate, apply/rebuild) stays on
-    // st; the restore chain (sort by (u,v), heads, restore) runs on st2.  The
-    // restore waits for validation so that an invalid batch mutates nothing.
-    cudaEventRecord(h->ev_fork, st);
-    cudaStreamWaitEvent(h->st2, h->ev_fork, 0);
-    cudaStream_t s2 = h->st2;
-    int wv = radix_sort_pairs(b.kv[0], b.ov[0], b.kv[1], b.ov[1], N, h->shifts, h->npasses,
-                              b.hist, st, &launches);
-    int wu = radix_sort_pairs(b.ku[0], b.ou[0], b.ku[1], b.ou[1], N, h->shifts, h->npasses,
-                              b.hist2, s2, &launches);
-    const uint64_t* kv = b.kv[wv];
-    const uint64_t* ku = b.ku[wu];
-    cudaMemsetAsync(b.claim, 0, sizeof(uint32_t) * N, st);
-    launch_heads(kv, b.ov[wv], N, b.rnv, b.vheads, &h->d_ctl->st.n_vheads, st, &launches);
-    launch_heads(ku, b.ou[wu], N, b.rnu, b.uheads, &h->d_ctl->st.n_uheads, s2, &launches);
-    // a1: graph store
-    launch_store_validate(dg, kv, N, b, h->vb, h->d_ctl, h->force_rebuild ? 1 : 0, st, &launches);
-    cudaEventRecord(h->ev_valid, st);
-    launch_store_apply(dg, kv, N, b, h->d_ctl, st, &launches);
-    StoreParams sp{h->slack, h->min_cap, h->pool_cap[h->active ^ 1u]};
-    launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches);
-    launch_seg_cleanup(kv, N, b, h->vb, h->d_ctl, st, &launches);
+    if (h->mode == PPR_MODE_ASYNC && h->push_enabled) {
+        rs = ensure_ring(h);
+        if (rs != PPR_OK) return rs;
+    }
+    if (use_graph) {  // one graph per batch shape, replayed
+        const GraphKey key{n_ins, n_del, h->push_enabled, h->mode, h->max_iters, h->timing,
+                           h->force_rebuild, h->buf_epoch, h->pool_cap[0], h->pool_cap[1],
+                           (const void*)h->d_pool[0], (const void*)h->d_pool[1]};
+        if (!h->gexec || !(key == h->gkey)) {
+            if (h->gexec) cudaGraphExecDestroy(h->gexec), h->gexec = nullptr;
+            cudaGraph_t graph = nullptr;
+            uint32_t glaunches = 0;
+            cudaError_t e = cudaStreamBeginCapture(st, cudaStreamCaptureModeThreadLocal);
+            ppr_status ers = PPR_OK;
+            if (e == cudaSuccess) ers = enqueue_batch(h, is, id, n_ins, ds, dd, n_del, N, &glaunches);
+            cudaError_t e2 = cudaStreamEndCapture(st, &graph);
+            if (e == cudaSuccess) e = e2;
+            if (e == cudaSuccess && ers == PPR_OK) e = cudaGraphInstantiate(&h->gexec, graph, 0);
+            if (graph) cudaGraphDestroy(graph);
+            if (e != cudaSuccess || ers != PPR_OK) {  // capture unsupported: run the stream path
+                cudaGetLastError();
+                h->gexec = nullptr;
+                h->graphs = false;
+                set_err(h, "graph capture failed (%s); using stream launches", cudaGetErrorString(e));
+                h->poisoned = false;
+            } else {
+                h->gkey = key;
+                h->glaunches = glaunches;
+            }
+        }
+        if (h->gexec) {
+            dbg_step("before graph launch");
+            cudaError_t e = cudaGraphLaunch(h->gexec, st);
+            if (e != cudaSuccess) return cuda_fail(h, e, "cudaGraphLaunch");
+            launches = h->glaunches;
+        } else {
+            rs = enqueue_batch(h, is, id, n_ins, ds, dd, n_del, N, &launches);
+            if (rs != PPR_OK) return rs;
+        }
+    } else {
+        rs = enqueue_batch(h, is, id, n_ins, ds, dd, n_del, N, &launches);
+        if (rs != PPR_OK) return rs;
+    }
+    // store and restore (two streams, joined) are timed together; the push is
+    // one cooperative launch between its own events on the handle's stream
     record(h, 1);
-    // a2: restore (after validation)
-    cudaStreamWaitEvent(s2, h->ev_valid, 0);
-    launch_restore(dg, ku, N, b, h->vb, h->d_ctl, s2, &launches);
-    cudaEventRecord(h->ev_join, s2);
-    cudaStreamWaitEvent(st, h->ev_join, 0);  // join
     record(h, 2);
-    // a3-a6: push
     if (h->push_enabled) {
         PushArgs a = push_args(h);
         a.seed_v = h->vb.touched;
         a.n_seed_v_dev = &h->d_ctl->st.n_touched;
         rs = run_push(h, a, &launches);
+        dbg_step("push");
         if (rs != PPR_OK) return rs;
     }
     record(h, 3);

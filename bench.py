@@ -37,8 +37,12 @@ import numpy as np
 ROOT = os.path.dirname(os.path.abspath(__file__))
 sys.path.insert(0, ROOT)
 
-# algorithmic bytes per unit
+# algorithmic bytes per unit: a pushed edge is
+# 24 B = 8 B of walk (v id + d_out(v)) + 16 B of R(v) read+write.  The shared
+# multi-source kernel walks an in-arc once per (source group, arc), so its
+# bytes are 8 per walked arc + 16 per (source, arc) propagation.
 B_EDGE, B_VERTEX, B_ARC = 24, 52, 56
+B_WALK, B_PROP = 8, 16
 
 
 def parse():
@@ -310,8 +314,8 @@ def run_ours(args):
     if und:
         deg = deg + np.bincount(win_np[1], minlength=cfg["n"])
     my_srcs = D.partition_sources(srcs_all, deg, ws, rank)
-    if args.mode == "auto":  # measured: Opt best single-source, EAGER_SCAN 2.4x better multi-source
-        args.mode = "opt" if len(my_srcs) == 1 else "scan"
+    if args.mode == "auto":  # measured: Opt best single-source, SHARED for several sources per rank
+        args.mode = "opt" if len(my_srcs) == 1 else "shared"
 
     t0 = time.perf_counter()
     h = ppr.Ppr(cfg["n"], win_np[0], win_np[1], my_srcs, alpha=0.15, eps=eps, mode=args.mode,
@@ -400,6 +404,7 @@ def run_ours(args):
     push_ms = sum(s["ms_push"] for s in stats)
     edges_r0 = sum(s["pushed_edges"] for s in stats)
     verts_r0 = sum(s["pushes"] for s in stats)
+    walks_r0 = sum(s["walk_edges"] for s in stats)
     edges, verts, launches = D.sum_over_ranks(
         [edges_r0, verts_r0, sum(s["kernel_launches"] for s in stats)], device=dev)
     dev_bytes = h.device_bytes
@@ -414,7 +419,7 @@ def run_ours(args):
     e2e_value = S * upd * len(e2e_ms) / (T_e2e / 1e3) if e2e_ms else None
     peak, peak_kind = measured_peak()
     # dominant kernel: the persistent push (one launch per step), rank 0's launches
-    bytes_per_launch = (B_EDGE * edges_r0 + B_VERTEX * verts_r0) / steps
+    bytes_per_launch = (B_WALK * walks_r0 + B_PROP * edges_r0 + B_VERTEX * verts_r0) / steps
     push_ms_avg = push_ms / steps
     achieved = bytes_per_launch / (push_ms_avg / 1e3) / 1e9 if push_ms_avg > 0 else 0.0
     traffic = profile_traffic(args.workload) if S == 1 else None
@@ -446,6 +451,7 @@ def run_ours(args):
             "pushed_edges_per_s": edges / (T / 1e3),
             "pushes_per_step": verts / steps / S,
             "pushed_edges_per_step": edges / steps / S,
+            "walk_edges_per_step_rank0": walks_r0 / steps,
             "iters_per_step": sum(s["iters_pos"] + s["iters_neg"] for s in stats) / steps,
             "rebuilds": sum(s["rebuilt"] for s in stats),
             "atomics_per_s_rank0": (edges_r0 + verts_r0) / (push_ms / 1e3) if push_ms else None,

@@ -72,10 +72,15 @@ enum {
     PPR_MODE_ASYNC = 4,     /* Alg 4's operations without rounds: asynchronous ring worklist
                                (any push order is valid by Lemma 1; DESIGN.md K-ASYNC);
                                iters_pos/iters_neg are reported as 0 */
-    PPR_MODE_EAGER_SCAN = 5 /* eager propagation; residual updates are fire-and-forget
+    PPR_MODE_EAGER_SCAN = 5, /* eager propagation; residual updates are fire-and-forget
                                reductions that mark touched vertices in a bitmap, and each
                                round's frontier comes from a warp-ballot/scan compaction of
                                that bitmap (DESIGN.md K-SCAN) */
+    PPR_MODE_SHARED = 6     /* multi-source: shared-adjacency push.  A frontier entry is a
+                               (vertex, group of 32 sources); one warp reads N_in(u) once and
+                               every lane pushes its own source's residual onto the shared
+                               [n][S] row (coalesced reductions); bitmap dedup + compaction as
+                               in EAGER_SCAN (DESIGN.md K-SHARED).  Any S >= 1; arrays layout */
 };
 
 /* Graph for ppr_create: m arcs src[i] -> dst[i] on [0, n) (host pointers).
@@ -118,6 +123,9 @@ typedef struct {
     uint64_t h2d_bytes, d2h_bytes;  /* host<->device bytes this call copied */
     float ms_total;                 /* CUDA-event time of the call on the stream */
     float ms_store, ms_restore, ms_push; /* per phase (0 if timing disabled) */
+    uint64_t walk_edges;            /* in-arc reads of the push: PPR_MODE_SHARED walks N_in(u) once
+                                       per (source group, u), so walk_edges <= pushed_edges;
+                                       other modes: = pushed_edges */
 } ppr_batch_stats;
 
 /* Creates a handle: builds the slab store for g, sets P_s = 0 and R_s = e_s

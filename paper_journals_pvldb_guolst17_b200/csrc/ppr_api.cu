@@ -267,6 +267,7 @@ void fill_stats(ppr_ctx* h, ppr_batch_stats* s, uint32_t launches, bool timed,
     s->iters_neg = c.iters[1];
     s->pushes = c.pushes;
     s->pushed_edges = c.pushed_edges;
+    s->walk_edges = h->mode == PPR_MODE_SHARED ? c.walk_edges : c.pushed_edges;
     s->max_frontier = c.max_frontier;
     s->touched = (uint64_t)c.n_touched * h->S;
     s->num_arcs = h->m;
@@ -552,7 +553,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     o.min_cap = 4;
     o.relabel = -1;
     if (opts) o = *opts;
-    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_EAGER_SCAN || !(o.slack >= 0.0) ||
+    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_SHARED || !(o.slack >= 0.0) ||
         o.min_cap == 0)
         return PPR_EINVAL;
 
@@ -604,7 +605,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     // Default: arrays (R + d_out = 12 B/vertex stay L2-resident, see ppr_internal.cuh);
     // PPR_LAYOUT=packed selects the 32-byte records for experiments.
     const char* lay = getenv("PPR_LAYOUT");
-    const bool packed = lay && !strcmp(lay, "packed") && h->S == 1 && pool_bound < 4.0e9;
+    const bool packed = lay && !strcmp(lay, "packed") && h->S == 1 && o.mode != PPR_MODE_SHARED && pool_bound < 4.0e9;
     bool ok = packed ? dalloc(h, &h->d_rec, h->n) == cudaSuccess
                      : (dalloc(h, &h->d_hot, Sn + (h->n + 1) / 2 + 32) == cudaSuccess &&
                         dalloc(h, &h->d_slab, h->n) == cudaSuccess &&
@@ -814,7 +815,8 @@ ppr_status ppr_set_option(ppr_ctx* h, int key, int64_t value) {
     if (h->poisoned) return PPR_EPOISONED;
     switch (key) {
         case PPR_OPT_MODE:
-            if (value < PPR_MODE_OPT || value > PPR_MODE_EAGER_SCAN) return PPR_EINVAL;
+            if (value < PPR_MODE_OPT || value > PPR_MODE_SHARED) return PPR_EINVAL;
+            if (value == PPR_MODE_SHARED && h->d_rec) return PPR_EINVAL;  // arrays layout only
             h->mode = (int)value;
             return PPR_OK;
         case PPR_OPT_PUSH: h->push_enabled = value != 0; return PPR_OK;

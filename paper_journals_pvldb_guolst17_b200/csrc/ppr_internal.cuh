@@ -53,6 +53,7 @@ struct DevStats {
     long long arc_delta;       // net change of the arc count this batch
     unsigned int n_big;        // vertices copied warp-wide in a rebuild
     unsigned int pad0;
+    unsigned long long walk_edges; // in-arc walks (SHARED: one per (source group, arc))
 };
 
 // A counter alone on its 128-byte line: the per-round counters, the tile

@@ -878,6 +878,7 @@ cudaError_t launch_layout(int mode, const PushArgs& a, int num_sms, cudaStream_t
 }  // namespace
 
 cudaError_t launch_push(int mode, const PushArgs& a, int num_sms, cudaStream_t st) {
+    if (mode == 6 /* PPR_MODE_SHARED */) return a.g.rec ? cudaErrorInvalidValue : launch_push_ms(a, num_sms, st);
     return a.g.rec ? launch_layout<true>(mode, a, num_sms, st)
                    : launch_layout<false>(mode, a, num_sms, st);
 }

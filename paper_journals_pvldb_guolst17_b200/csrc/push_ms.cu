@@ -1,0 +1,409 @@
+// push_ms.cu -- shared-adjacency multi-source push (PPR_MODE_SHARED; SURVEY
+// 8(f) NEXT-3, steps a3-a6 of the hot path for S > 1 sources).
+//
+// The S sources of a handle are independent unit-vector problems
+// over one graph, so their pushes walk the same in-lists.  This kernel makes
+// a frontier entry a (group, vertex) pair, where a group is 32 consecutive
+// source columns of the vertex-major [n][S] residual array, and gives every
+// lane of a warp one source of the group:
+//   * Alg 4 line 10 (eager read): lane l reads R_{32g+l}(u) with
+//     a relaxed load -- one coalesced 256-byte row read per entry -- and the
+//     lanes whose residual meets pushCond form the entry's push mask.
+//   * Alg 4 lines 20-21 (self-update): P(u) += a r, R(u) -= r for the masked
+//     lanes, as fire-and-forget reductions (coalesced).
+//   * Alg 4 lines 11-13 (propagation): N_in(u) is read ONCE for the whole
+//     group; for every v the masked lanes add (1-a) r_l / d(v) to
+//     R_{32g+l}(v): one warp-wide reduction onto one contiguous row segment
+//     instead of up to 32 random single-word atomics.
+//   * Frontier generation (north_star "bitmap dedup plus warp-ballot/scan
+//     compaction"): every changed (v, g) is marked in a bitmap; after a grid
+//     barrier the bitmap is compacted into the next frontier.  Whether an
+//     entry pushes any lane is decided when it is processed (the row read
+//     above), so the scan is pure bit compaction.
+// Termination and correctness follow DESIGN.md K-SCAN: every residual change
+// marks its (v, g), the next round re-reads every marked row after the
+// barrier, so a round that finds no lane meeting pushCond changes nothing
+// and the phase ends with -eps <= R <= eps everywhere.  Each entry is in a
+// frontier at most once per round (the bitmap deduplicates), so no residual
+// mass is pushed twice.  Seeding: the touched vertices (every group), the
+// sources (create) or every (v, g) (ppr_push) are marked and compacted.
+//
+// The increment is ((1-a) r) * (1/d(v)): the reciprocal is computed once per
+// edge and shared by the 32 lanes (reading R-RCP; the oracle
+// divides, the two differ by at most one rounding per increment, far inside
+// the invariant tolerance R18).
+#include "block_scan.cuh"
+#include "push.cuh"
+
+namespace ppr {
+
+namespace {
+
+constexpr int PT = PUSH_THREADS;
+constexpr int NW = PT / 32;
+constexpr int MT = 64;    // frontier entries per CTA tile
+constexpr int QW = 256;   // per-warp queue slice (entries)
+
+struct MsSmem {
+    double w[MT][32];                 // (1-a) r of every lane of every entry (0: lane idle)
+    unsigned long long off[MT];       // slab offset of each entry
+    uint32_t scan[2 * MT];            // exclusive prefix of the entries' walk lengths
+    uint32_t grp[MT];                 // source group of each entry
+    uint32_t len[MT];                 // walk length (in-degree, or 0 if no lane pushes)
+    unsigned long long q[NW][QW];     // per-warp enqueue slices
+    unsigned int wq[NW];
+    unsigned long long gbase;
+    unsigned long long next;
+    unsigned long long cround;
+    unsigned int chunk;
+    uint32_t E;
+};
+
+struct MsCtx {
+    const uint32_t* pool;
+    unsigned long long* Fout;
+    unsigned long long* cnt_out;
+    uint32_t qn;
+    unsigned long long pushes;     // (source, vertex) self-updates
+    unsigned long long edges;      // (source, arc) propagations
+    unsigned long long walks;      // (group, arc) walks
+};
+
+__device__ __forceinline__ unsigned lane() { return threadIdx.x & 31u; }
+__device__ __forceinline__ unsigned warp() { return threadIdx.x >> 5; }
+
+__device__ __forceinline__ void warp_flush(MsSmem& s, MsCtx& c) {
+    if (c.qn == 0) return;  // warp-uniform
+    unsigned long long base = 0;
+    if (lane() == 0) base = atomicAdd(c.cnt_out, (unsigned long long)c.qn);
+    base = __shfl_sync(0xffffffffu, base, 0);
+    for (uint32_t i = lane(); i < c.qn; i += 32) __stcg(&c.Fout[base + i], s.q[warp()][i]);
+    __syncwarp();
+    c.qn = 0;
+}
+
+__device__ __forceinline__ void warp_enqueue(MsSmem& s, MsCtx& c, bool flag, unsigned long long e) {
+    if (c.qn + 32 > QW) {
+        __syncwarp();
+        warp_flush(s, c);
+    }
+    const unsigned b = __ballot_sync(0xffffffffu, flag);
+    if (flag) s.q[warp()][c.qn + __popc(b & ((1u << lane()) - 1u))] = e;
+    c.qn += __popc(b);
+}
+
+__device__ __forceinline__ void block_flush(MsSmem& s, MsCtx& c) {
+    const unsigned w = warp();
+    __syncwarp();
+    if (lane() == 0) s.wq[w] = c.qn;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        unsigned long long tot = 0;
+        for (int i = 0; i < NW; i++) {
+            const unsigned x = s.wq[i];
+            s.wq[i] = (unsigned)tot;
+            tot += x;
+        }
+        s.gbase = tot ? atomicAdd(c.cnt_out, tot) : 0ull;
+    }
+    __syncthreads();
+    const unsigned long long base = s.gbase + s.wq[w];
+    for (uint32_t i = lane(); i < c.qn; i += 32) __stcg(&c.Fout[base + i], s.q[w][i]);
+    c.qn = 0;
+    __syncthreads();
+}
+
+// Marks (v, g).  The test reads the word at L2 (never a stale L1 copy: the
+// scan clears words between rounds), so a set bit is only skipped when it is
+// really set.
+__device__ __forceinline__ void mark(uint32_t* bitmap, unsigned long long bit) {
+    const uint32_t m = 1u << (bit & 31u);
+    uint32_t* p = &bitmap[bit >> 5];
+    if (!(__ldcg(p) & m)) atomicOr(p, m);
+}
+
+// largest i with scan[i] <= e (scan[T..] hold 0xFFFFFFFF)
+__device__ __forceinline__ int owner_of(const uint32_t* scan, uint32_t e, int top) {
+    int lo = 0;
+    for (int step = top; step > 0; step >>= 1)
+        if (scan[lo + step] <= e) lo += step;
+    return lo;
+}
+
+// ---------------------------------------------------------------- one tile
+
+template <bool POS>
+__device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, uint32_t SG,
+                                        const unsigned long long* Fin, uint64_t C, uint64_t base,
+                                        uint32_t T, int top) {
+    const unsigned L = lane(), w = warp();
+    const uint32_t S = a.g.S;
+    const double eps = a.g.eps, alpha = a.g.alpha;
+    const unsigned long long pol_keep = l2_keep(), pol_stream = l2_stream();
+    // Phase A: one warp per entry -- eager row read, push mask, self-update
+    for (uint32_t j = w; j < T; j += NW) {
+        const uint64_t idx = base + j;
+        const bool ve = idx < C;  // warp-uniform
+        const unsigned long long ent = ve ? __ldcg(&Fin[idx]) : 0ull;
+        const uint32_t g = (uint32_t)(ent >> 32), u = (uint32_t)ent;
+        ulonglong2 sl = make_ulonglong2(0, 0);
+        if (ve && L == 0) sl = ld_u64x2_pol(&a.g.slab[u], pol_stream);  // Slab {off, len|cap}
+        const uint32_t sidx = g * 32 + L;
+        const bool lok = ve && sidx < S;
+        double* ru = a.g.R + (size_t)u * S + sidx;
+        const double r = lok ? ld_relaxed_f64(ru) : 0.0;
+        const bool p = lok && push_cond<POS>(r, eps);
+        const unsigned mask = __ballot_sync(0xffffffffu, p);
+        if (p) {
+            red_add_pol(ru, -r, pol_keep);
+            red_add_pol(a.g.P + (size_t)u * S + sidx, __dmul_rn(alpha, r), pol_stream);
+        }
+        s.w[j][L] = p ? __dmul_rn(1.0 - alpha, r) : 0.0;
+        if (L == 0) {
+            const uint32_t len = mask ? (uint32_t)sl.y : 0u;
+            s.len[j] = len;
+            s.off[j] = sl.x;
+            s.grp[j] = g;
+            if (mask) {
+                mark(a.bitmap, (unsigned long long)u * SG + g);  // u's row changed
+                const unsigned k = __popc(mask);
+                c.pushes += k;
+                c.edges += (unsigned long long)k * len;
+                c.walks += len;
+            }
+        }
+    }
+    __syncthreads();
+    // exclusive scan of the T walk lengths (warp 0, two entries per lane)
+    if (w == 0) {
+        const uint32_t a0 = 2 * L < T ? s.len[2 * L] : 0u;
+        const uint32_t a1 = 2 * L + 1 < T ? s.len[2 * L + 1] : 0u;
+        uint32_t inc = a0 + a1;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const uint32_t y = __shfl_up_sync(0xffffffffu, inc, o);
+            if (L >= (unsigned)o) inc += y;
+        }
+        const uint32_t ex = inc - a0 - a1;
+        s.scan[2 * L] = 2 * L < T ? ex : 0xFFFFFFFFu;
+        s.scan[2 * L + 1] = 2 * L + 1 < T ? ex + a0 : 0xFFFFFFFFu;
+        s.scan[2 * L + MT] = 0xFFFFFFFFu;
+        s.scan[2 * L + 1 + MT] = 0xFFFFFFFFu;
+        if (L == 31) {
+            s.E = inc;
+            s.chunk = 0;
+        }
+    }
+    __syncthreads();
+    const uint32_t E = s.E;
+    // Phase B: warps claim 32-arc chunks of the tile's walk; lane k loads arc k
+    // (v, d(v), 1/d(v)) and marks (v, g), then the warp applies the 32 arcs one
+    // by one, every lane adding its source's increment to the shared row
+    while (true) {
+        uint32_t cb = 0;
+        if (L == 0) cb = atomicAdd(&s.chunk, 1u);
+        cb = __shfl_sync(0xffffffffu, cb, 0);
+        if (cb * 32 >= E) break;
+        const uint32_t e = cb * 32 + L;
+        const bool ok = e < E;
+        int j = 0;
+        uint32_t v = 0, d = 1;
+        if (ok) {
+            j = owner_of(s.scan, e, top);
+            v = ld_u32_pol(&c.pool[s.off[j] + (e - s.scan[j])], pol_stream);
+            d = ld_u32_pol(&a.g.dout[v], pol_keep);
+            mark(a.bitmap, (unsigned long long)v * SG + s.grp[j]);
+        }
+        const double rd = __drcp_rn((double)d);
+        const uint32_t nk = E - cb * 32 < 32 ? E - cb * 32 : 32;
+        for (uint32_t k = 0; k < nk; k++) {
+            const uint32_t vk = __shfl_sync(0xffffffffu, v, k);
+            const int jk = __shfl_sync(0xffffffffu, j, k);
+            const double rk = __shfl_sync(0xffffffffu, rd, k);
+            const double wl = s.w[jk][L];
+            if (wl != 0.0)
+                red_add_pol(a.g.R + (size_t)vk * S + s.grp[jk] * 32 + L, __dmul_rn(wl, rk), pol_keep);
+        }
+    }
+    __syncthreads();  // smem of this tile is reused by the next
+}
+
+// every CTA takes tiles of T entries (first statically, the rest by claims)
+template <bool POS>
+__device__ __forceinline__ void ms_round(MsSmem& s, MsCtx& c, const PushArgs& a, uint32_t SG,
+                                         const unsigned long long* Fin, uint64_t C,
+                                         unsigned long long* tc) {
+    const uint64_t per = (C + gridDim.x - 1) / gridDim.x;
+    uint32_t T = (uint32_t)((per + NW - 1) / NW * NW);
+    if (T > MT) T = MT;
+    if (T < NW) T = NW;
+    int top = 1;
+    while (top * 2 < (int)T) top <<= 1;
+    const uint64_t ntiles = (C + T - 1) / T;
+    uint64_t t = blockIdx.x;
+    while (t < ntiles) {
+        ms_tile<POS>(s, c, a, SG, Fin, C, t * T, T, top);
+        if (ntiles <= gridDim.x) break;
+        if (threadIdx.x == 0) s.next = atomicAdd(tc, 1ull) + gridDim.x;
+        __syncthreads();
+        t = s.next;
+        __syncthreads();
+    }
+}
+
+// compacts the marked (v, g) bits into the frontier (bit = v * SG + g) and
+// clears them; emitted entries are sorted by vertex within a warp's words
+__device__ __forceinline__ void ms_scan(MsSmem& s, MsCtx& c, const PushArgs& a, uint32_t SG) {
+    const uint64_t nwords = ((uint64_t)SG * a.g.n + 31) / 32;
+    const uint64_t gw = (uint64_t)blockIdx.x * NW + warp(), nw = (uint64_t)gridDim.x * NW;
+    for (uint64_t w0 = gw * 32; w0 < nwords; w0 += nw * 32) {
+        const uint64_t wi = w0 + lane();
+        uint32_t word = wi < nwords ? __ldcg(&a.bitmap[wi]) : 0u;
+        if (word) __stcg(&a.bitmap[wi], 0u);
+        while (__any_sync(0xffffffffu, word != 0)) {
+            bool enq = false;
+            unsigned long long ent = 0;
+            if (word) {
+                const int b = __ffs(word) - 1;
+                word &= word - 1;
+                const uint64_t bit = wi * 32 + b;
+                ent = ((bit % SG) << 32) | (bit / SG);
+                enq = true;
+            }
+            warp_enqueue(s, c, enq, ent);
+        }
+    }
+}
+
+// marks the phase's seeds
+__device__ __forceinline__ void ms_seed(const PushArgs& a, uint32_t SG) {
+    const uint64_t stride = (uint64_t)gridDim.x * PT;
+    const uint64_t t0 = (uint64_t)blockIdx.x * PT + threadIdx.x;
+    if (a.seed_all) {
+        const uint64_t nbits = (uint64_t)SG * a.g.n, nwords = (nbits + 31) / 32;
+        for (uint64_t wi = t0; wi < nwords; wi += stride) {
+            const uint64_t rem = nbits - wi * 32;
+            a.bitmap[wi] = rem >= 32 ? 0xFFFFFFFFu : ((1u << rem) - 1u);
+        }
+    } else if (a.seed_v) {
+        const uint64_t nv = *a.n_seed_v_dev;
+        for (uint64_t k = t0; k < nv * SG; k += stride)
+            mark(a.bitmap, (unsigned long long)a.seed_v[k / SG] * SG + (k % SG));
+    } else {
+        for (uint64_t k = t0; k < a.n_seed_e; k += stride) {
+            const unsigned long long ent = a.seed_e[k];
+            mark(a.bitmap, (unsigned long long)(uint32_t)ent * SG + (uint32_t)(ent >> 32) / 32);
+        }
+    }
+}
+
+template <bool POS>
+__device__ __forceinline__ void ms_phase(MsSmem& s, MsCtx& c, const PushArgs& a, uint32_t SG,
+                                         unsigned& it) {
+    DevCtl* ctl = a.ctl;
+    const int ph = POS ? 0 : 1;
+    ms_seed(a, SG);
+    grid_sync(ctl);
+    c.Fout = a.F[it & 1];
+    c.cnt_out = &ctl->fcount[it % 3].v;
+    ms_scan(s, c, a, SG);
+    block_flush(s, c);
+    grid_sync(ctl);
+    uint32_t pit = 0;
+    while (true) {
+        if (threadIdx.x == 0) s.cround = *(volatile unsigned long long*)&ctl->fcount[it % 3].v;
+        __syncthreads();
+        const uint64_t C = s.cround;
+        if (blockIdx.x == 0 && threadIdx.x == 0) {
+            ctl->fcount[(it + 2) % 3].v = 0;
+            ctl->tilectr[(it + 2) % 3].v = 0;
+            if (C > 0 && !(a.max_iters && pit >= a.max_iters)) {
+                ctl->st.iters[ph]++;
+                atomicMax(&ctl->st.max_frontier, (unsigned long long)C);
+            }
+            if (C > 0 && pit >= a.iter_cap) atomicCAS(&ctl->st.err, KERR_OK, KERR_NOCONV);
+        }
+        if (C == 0 || (a.max_iters && pit >= a.max_iters) || pit >= a.iter_cap) break;
+        const unsigned long long* Fin = a.F[it & 1];
+        c.Fout = a.F[(it + 1) & 1];
+        c.cnt_out = &ctl->fcount[(it + 1) % 3].v;
+        ms_round<POS>(s, c, a, SG, Fin, C, &ctl->tilectr[it % 3].v);
+        grid_sync(ctl);  // every reduction and mark of the round has landed
+        ms_scan(s, c, a, SG);
+        block_flush(s, c);
+        grid_sync(ctl);
+        it++;
+        pit++;
+    }
+    grid_sync(ctl);
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+        ctl->fcount[0].v = ctl->fcount[1].v = ctl->fcount[2].v = 0;
+        ctl->tilectr[0].v = ctl->tilectr[1].v = ctl->tilectr[2].v = 0;
+    }
+    grid_sync(ctl);
+}
+
+__global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_constant__ PushArgs a) {
+    __shared__ MsSmem s;
+    MsCtx c;
+    c.qn = 0;
+    c.pushes = c.edges = c.walks = 0;
+    if (*(volatile int*)&a.ctl->st.err != KERR_OK) return;  // earlier stage failed: uniform exit
+    c.pool = *(volatile unsigned*)&a.ctl->st.active_pool ? a.g.pool[1] : a.g.pool[0];
+    const uint32_t SG = (a.g.S + 31) / 32;
+    if (blockIdx.x == 0 && threadIdx.x == 0)
+        for (int i = 0; i < 3; i++) a.ctl->fcount[i].v = a.ctl->tilectr[i].v = 0;
+    grid_sync(a.ctl);
+    unsigned it = 0;
+    if (a.phases & 1) ms_phase<true>(s, c, a, SG, it);
+    if (a.phases & 2) ms_phase<false>(s, c, a, SG, it);
+    __shared__ unsigned long long s_red[3];
+    if (threadIdx.x < 3) s_red[threadIdx.x] = 0;
+    __syncthreads();
+    if (c.pushes) atomicAdd(&s_red[0], c.pushes);
+    if (c.edges) atomicAdd(&s_red[1], c.edges);
+    if (c.walks) atomicAdd(&s_red[2], c.walks);
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        if (s_red[0]) atomicAdd(&a.ctl->st.pushes, s_red[0]);
+        if (s_red[1]) atomicAdd(&a.ctl->st.pushed_edges, s_red[1]);
+        if (s_red[2]) atomicAdd(&a.ctl->st.walk_edges, s_red[2]);
+    }
+}
+
+}  // namespace
+
+cudaError_t launch_push_ms(const PushArgs& a, int num_sms, cudaStream_t st) {
+    static int blocks_per_sm = 0;
+    if (blocks_per_sm == 0) {
+        cudaError_t e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push_ms, PT, 0);
+        if (e != cudaSuccess) return e;
+        if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
+        if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
+    }
+    PushArgs copy = a;
+    void* args[] = {&copy};
+    cudaLaunchConfig_t cfg{};
+    cfg.gridDim = dim3(num_sms * blocks_per_sm);
+    cfg.blockDim = dim3(PT);
+    cfg.stream = st;
+    cudaLaunchAttribute at[2];
+    int na = 0;
+    at[na].id = cudaLaunchAttributeCooperative;
+    at[na].val.cooperative = 1;
+    na++;
+    if (a.l2_bytes) {
+        at[na].id = cudaLaunchAttributeAccessPolicyWindow;
+        at[na].val.accessPolicyWindow.base_ptr = a.l2_base;
+        at[na].val.accessPolicyWindow.num_bytes = a.l2_bytes;
+        at[na].val.accessPolicyWindow.hitRatio = a.l2_hit;
+        at[na].val.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
+        at[na].val.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
+        na++;
+    }
+    cfg.attrs = at;
+    cfg.numAttrs = na;
+    return cudaLaunchKernelExC(&cfg, (const void*)k_push_ms, args);
+}
+
+}  // namespace ppr

@@ -20,9 +20,10 @@ LIB_PATH = os.path.join(_PKG, "libppr.so")
 PPR_OK, PPR_EINVAL, PPR_ERANGE, PPR_ENOENT, PPR_ENOMEM, PPR_ECUDA, PPR_EPOISONED, PPR_ENOCONV = \
     0, -1, -2, -3, -4, -5, -6, -7
 MEM_HOST, MEM_DEVICE = 0, 1
-MODE_OPT, MODE_EAGER, MODE_DUPDETECT, MODE_VANILLA, MODE_ASYNC, MODE_EAGER_SCAN = 0, 1, 2, 3, 4, 5
+MODE_OPT, MODE_EAGER, MODE_DUPDETECT, MODE_VANILLA, MODE_ASYNC, MODE_EAGER_SCAN, MODE_SHARED = \
+    0, 1, 2, 3, 4, 5, 6
 MODES = {"opt": MODE_OPT, "eager": MODE_EAGER, "dupdetect": MODE_DUPDETECT, "vanilla": MODE_VANILLA,
-         "async": MODE_ASYNC, "scan": MODE_EAGER_SCAN}
+         "async": MODE_ASYNC, "scan": MODE_EAGER_SCAN, "shared": MODE_SHARED}
 OPT_MODE, OPT_PUSH, OPT_MAX_ITERS, OPT_TIMING, OPT_FORCE_REBUILD = 1, 2, 3, 4, 5
 
 
@@ -45,7 +46,7 @@ class BatchStats(ctypes.Structure):
                 ("kernel_launches", ctypes.c_uint32), ("h2d_bytes", ctypes.c_uint64),
                 ("d2h_bytes", ctypes.c_uint64), ("ms_total", ctypes.c_float),
                 ("ms_store", ctypes.c_float), ("ms_restore", ctypes.c_float),
-                ("ms_push", ctypes.c_float)]
+                ("ms_push", ctypes.c_float), ("walk_edges", ctypes.c_uint64)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}

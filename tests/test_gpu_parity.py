@@ -19,7 +19,7 @@ from tests import golden_figs as G
 
 pytestmark = pytest.mark.gpu
 
-MODES = ["opt", "eager", "dupdetect", "vanilla", "async", "scan"]
+MODES = ["opt", "eager", "dupdetect", "vanilla", "async", "scan", "shared"]
 
 
 def _fig_gpu(mode="vanilla", max_iters=0):
@@ -169,6 +169,47 @@ def test_tiny_config_eps_1e9_l1_gate():
 
 def test_tiny_config_multi_source():
     _run_stream("tiny", "opt", slides=6, sources=4, check_every=3)
+
+
+@pytest.mark.parametrize("sources", [3, 32, 40, 70])
+def test_tiny_config_multi_source_shared(sources):
+    # PPR_MODE_SHARED (DESIGN.md K-SHARED): one full group, partial groups
+    # (S = 40: lanes 8..31 of group 1 idle), several groups; every source of
+    # every batch against the sequential oracle
+    _run_stream("tiny", "shared", slides=5, sources=sources, check_every=1)
+
+
+def test_tiny_config_multi_source_shared_relabelled_rebuild():
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 36)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=1e-8, mode="shared", relabel=1)
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, 1e-8)
+    o.push(oracle.SEQ)
+    h.set_option(ppr.OPT_FORCE_REBUILD, 1)
+    for t in range(3):
+        b = st.next_batch()
+        stt = h.apply_batch(*b)
+        assert stt["rebuilt"] == 1 and stt["walk_edges"] <= stt["pushed_edges"]
+        o.apply(*b)
+        for i, s in enumerate(srcs):
+            _check_batch_state(h, o, i, int(s), 1e-8, f"shared rebuild slide {t} source {i}")
+
+
+def test_shared_full_scan_push_matches_static():
+    # ppr_reset + ppr_push (seed_all) recomputes static PPR for all sources
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 33)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=1e-8, mode="shared")
+    h.reset()
+    h.push()
+    gs, gd = h.export_edges()
+    for i in (0, 17, 32):
+        P, R = h.query(i)
+        assert exact.terminated(R, 1e-8)
+        Pstar = exact.ppr_power(cfg["n"], gs, gd, int(srcs[i]), 0.15)
+        assert np.max(np.abs(P - Pstar)) <= 1e-8 * (1 + 1e-6)
 
 
 def test_tiny_against_power_iteration():
@@ -373,3 +414,36 @@ def test_orkut_full_size_properties():
     gs, gd = h.export_edges()
     ok, worst = exact.invariant_ok(cfg["n"], gs, gd, int(s), 0.15, P, R)
     assert ok, worst
+
+
+def test_lj_multi_source_shared_full_size():
+    """configs[4] shape (LJ-shaped, hub-band sources) in the bench's launch
+    configuration for several sources per rank (PPR_MODE_SHARED, relabelled):
+    two 10^4+10^4 slides with S = 64; termination for every source, Eq. 2 for
+    sampled sources, and one source against the sequential oracle (every
+    vertex, L_inf <= 2 eps)."""
+    st, cfg = W.make_stream("lj")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 64)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=cfg["eps"], mode="shared")
+    k = 37  # the oracle follows one source of the second group
+    o = oracle.Oracle(cfg["n"], g0s, g0d, [srcs[k]], 0.15, cfg["eps"])
+    o.push(oracle.SEQ)
+    for t in range(2):
+        b = st.next_batch()
+        stats = h.apply_batch(*b)
+        o.apply(*b)
+        assert stats["walk_edges"] < stats["pushed_edges"]  # in-lists really shared
+    gs, gd = h.export_edges()
+    os_, od = o.export()
+    np.testing.assert_array_equal(gd, od)
+    np.testing.assert_array_equal(gs, os_)
+    for i in range(64):
+        P, R = h.query(i)
+        assert exact.terminated(R, cfg["eps"]), i
+        if i in (0, 31, 32, k, 63):
+            ok, worst = exact.invariant_ok(cfg["n"], gs, gd, int(srcs[i]), 0.15, P, R)
+            assert ok, (i, worst)
+        if i == k:
+            Po, _ = o.query(0)
+            assert np.max(np.abs(P - Po)) <= 2 * cfg["eps"]

@@ -59,6 +59,8 @@ def parse():
     p.add_argument("--ins", type=int, default=None)
     p.add_argument("--dele", type=int, default=None)
     p.add_argument("--seed", type=int, default=42)
+    p.add_argument("--band", type=int, default=None,
+                   help="sources drawn from the top-BAND out-degree vertices (default: the config's 1000)")
     p.add_argument("--no-cpu-baseline", action="store_true")
     p.add_argument("--cpu-budget-s", type=float, default=30.0)
     p.add_argument("--ref-budget-s", type=float, default=150.0)
@@ -180,6 +182,8 @@ def run_reference(args):
         over["ins"] = args.ins
     if args.dele is not None:
         over["dele"] = args.dele
+    if args.band is not None:
+        over["band"] = args.band
     st, cfg = W.make_stream(args.workload, seed=args.seed, **over)
     eps = args.eps or cfg["eps"]
     g0s, g0d = st.window()
@@ -262,6 +266,8 @@ def run_ours(args):
         over["ins"] = args.ins
     if args.dele is not None:
         over["dele"] = args.dele
+    if args.band is not None:
+        over["band"] = args.band
     cfg = dict(W.CONFIGS[args.workload])
     cfg.update(over)
     eps = args.eps or cfg["eps"]

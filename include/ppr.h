@@ -76,11 +76,18 @@ enum {
                                reductions that mark touched vertices in a bitmap, and each
                                round's frontier comes from a warp-ballot/scan compaction of
                                that bitmap (DESIGN.md K-SCAN) */
-    PPR_MODE_SHARED = 6     /* multi-source: shared-adjacency push.  A frontier entry is a
+    PPR_MODE_SHARED = 6,    /* multi-source: shared-adjacency push.  A frontier entry is a
                                (vertex, group of 32 sources); one warp reads N_in(u) once and
                                every lane pushes its own source's residual onto the shared
                                [n][S] row (coalesced reductions); bitmap dedup + compaction as
                                in EAGER_SCAN (DESIGN.md K-SHARED).  Any S >= 1; arrays layout */
+    PPR_MODE_SORTAGG = 7    /* Alg 3 rounds with sort-and-aggregate propagation instead of
+                               atomics (the alternative of P:433-442): pairs (v, (1-a)w_u/d(v))
+                               are radix-sorted by v and each run is added to R(v) in
+                               ascending-u order.  No atomics: bit-reproducible, and equal bit
+                               for bit to a sequential Alg 3 round loop over the sorted frontier
+                               when ids are not relabelled (ppr_opts.relabel = 0).  Host-driven
+                               rounds; arrays layout (DESIGN.md K-SORTAGG) */
 };
 
 /* Graph for ppr_create: m arcs src[i] -> dst[i] on [0, n) (host pointers).

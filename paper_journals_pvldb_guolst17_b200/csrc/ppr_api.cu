@@ -18,6 +18,7 @@
 #include <algorithm>
 #include <cmath>
 #include <cstdarg>
+#include <cstddef>
 #include <cstdio>
 #include <cstdlib>
 #include <cstring>
@@ -113,6 +114,7 @@ struct ppr_ctx {
     unsigned long long ring_cap = 0;
     unsigned long long* d_trace = nullptr;  // PPR_TRACE=1: per-round trace of the push
     uint32_t trace_cap = 0;
+    SortAgg* sa = nullptr;                  // PPR_MODE_SORTAGG scratch (grown on demand)
 };
 
 namespace {
@@ -409,6 +411,11 @@ void destroy_all(ppr_ctx* h) {
     if (h->st2) cudaStreamSynchronize(h->st2), cudaStreamDestroy(h->st2), h->st2 = nullptr;
     dfree(h, h->d_trace, 4ull * h->trace_cap + 8);
     dfree(h, h->d_ring, h->ring_cap);
+    if (h->sa) {
+        h->dev_bytes -= sortagg_bytes(h->sa);
+        sortagg_free(h->sa);
+        h->sa = nullptr;
+    }
     if (h->own_stream && h->st) cudaStreamDestroy(h->st);
     h->st = nullptr;
 }
@@ -425,7 +432,42 @@ ppr_status ensure_ring(ppr_ctx* h) {
     return PPR_OK;
 }
 
+// PPR_MODE_SORTAGG: host-driven rounds (push_sortagg.cu); the statistics the
+// persistent kernel would have accumulated are written into the control block
+ppr_status run_push_sortagg(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
+    cudaError_t e = cudaMemcpyAsync(h->h_ctl, &h->d_ctl->st, sizeof(DevStats), cudaMemcpyDeviceToHost, h->st);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(h->st);
+    if (e != cudaSuccess) return cuda_fail(h, e, "sortagg (control block)");
+    if (h->h_ctl->err != KERR_OK) return PPR_OK;  // an earlier stage failed: finish() maps it
+    SortAggStats out;
+    out.active_pool = h->h_ctl->active_pool;
+    const uint64_t before = sortagg_bytes(h->sa);
+    e = sortagg_push(&h->sa, a, a.seed_v ? h->h_ctl->n_touched : 0, h->st, &out, launches);
+    h->dev_bytes += sortagg_bytes(h->sa) - before;
+    if (e == cudaErrorMemoryAllocation) {
+        cudaGetLastError();
+        set_err(h, "out of device memory for the sort-and-aggregate pairs");
+        h->poisoned = true;
+        return PPR_ENOMEM;
+    }
+    if (e != cudaSuccess) return cuda_fail(h, e, "sortagg push");
+    struct {
+        unsigned long long pushes, edges, max_frontier;
+        unsigned iters[2];
+    } w{out.pushes, out.edges, out.max_frontier, {out.iters[0], out.iters[1]}};
+    static_assert(sizeof(w) == offsetof(DevStats, err), "DevStats prefix layout");
+    cudaMemcpyAsync(&h->d_ctl->st, &w, sizeof w, cudaMemcpyHostToDevice, h->st);
+    if (out.noconv) {
+        const int k = KERR_NOCONV;
+        cudaMemcpyAsync(&h->d_ctl->st.err, &k, sizeof k, cudaMemcpyHostToDevice, h->st);
+    }
+    e = cudaStreamSynchronize(h->st);
+    if (e != cudaSuccess) return cuda_fail(h, e, "sortagg stats");
+    return PPR_OK;
+}
+
 ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
+    if (h->mode == PPR_MODE_SORTAGG) return run_push_sortagg(h, a, launches);
     if (h->mode == PPR_MODE_ASYNC && !h->d_ring) {
         ppr_status rs = ensure_ring(h);
         if (rs != PPR_OK) return rs;
@@ -553,7 +595,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     o.min_cap = 4;
     o.relabel = -1;
     if (opts) o = *opts;
-    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_SHARED || !(o.slack >= 0.0) ||
+    if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_SORTAGG || !(o.slack >= 0.0) ||
         o.min_cap == 0)
         return PPR_EINVAL;
 
@@ -605,7 +647,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     // Default: arrays (R + d_out = 12 B/vertex stay L2-resident, see ppr_internal.cuh);
     // PPR_LAYOUT=packed selects the 32-byte records for experiments.
     const char* lay = getenv("PPR_LAYOUT");
-    const bool packed = lay && !strcmp(lay, "packed") && h->S == 1 && o.mode != PPR_MODE_SHARED && pool_bound < 4.0e9;
+    const bool packed = lay && !strcmp(lay, "packed") && h->S == 1 && o.mode != PPR_MODE_SHARED && o.mode != PPR_MODE_SORTAGG && pool_bound < 4.0e9;
     bool ok = packed ? dalloc(h, &h->d_rec, h->n) == cudaSuccess
                      : (dalloc(h, &h->d_hot, Sn + (h->n + 1) / 2 + 32) == cudaSuccess &&
                         dalloc(h, &h->d_slab, h->n) == cudaSuccess &&
@@ -815,8 +857,9 @@ ppr_status ppr_set_option(ppr_ctx* h, int key, int64_t value) {
     if (h->poisoned) return PPR_EPOISONED;
     switch (key) {
         case PPR_OPT_MODE:
-            if (value < PPR_MODE_OPT || value > PPR_MODE_SHARED) return PPR_EINVAL;
-            if (value == PPR_MODE_SHARED && h->d_rec) return PPR_EINVAL;  // arrays layout only
+            if (value < PPR_MODE_OPT || value > PPR_MODE_SORTAGG) return PPR_EINVAL;
+            if ((value == PPR_MODE_SHARED || value == PPR_MODE_SORTAGG) && h->d_rec)
+                return PPR_EINVAL;  // arrays layout only
             h->mode = (int)value;
             return PPR_OK;
         case PPR_OPT_PUSH: h->push_enabled = value != 0; return PPR_OK;

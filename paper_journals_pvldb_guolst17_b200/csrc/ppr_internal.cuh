@@ -205,6 +205,12 @@ __device__ __forceinline__ double atom_add_pol(double* a, double v, unsigned lon
                  : "=d"(r) : "l"(a), "d"(v), "l"(pol) : "memory");
     return r;
 }
+__device__ __forceinline__ double atom_exch_f64_pol(double* a, double v, unsigned long long pol) {
+    unsigned long long r;
+    asm volatile("atom.global.exch.L2::cache_hint.b64 %0, [%1], %2, %3;"
+                 : "=l"(r) : "l"(a), "l"(__double_as_longlong(v)), "l"(pol) : "memory");
+    return __longlong_as_double(r);
+}
 __device__ __forceinline__ void red_add_pol(double* a, double v, unsigned long long pol) {
     asm volatile("red.global.add.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(a), "d"(v), "l"(pol)
                  : "memory");

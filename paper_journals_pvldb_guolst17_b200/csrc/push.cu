@@ -54,6 +54,22 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_PUSH_U
 #define PPR_PUSH_U 2
 #endif
+// Opt self-update by exchange: r_u = atomicExch(R(u), 0) (DESIGN.md K-PUSH)
+// per-CTA time split of the trace (PPR_TRACE): compiled in only on request,
+// its counters would otherwise cost registers in every thread
+#ifndef PPR_PUSH_TIMESPLIT
+#define PPR_PUSH_TIMESPLIT 0
+#endif
+constexpr bool kTimeSplit = PPR_PUSH_TIMESPLIT;
+#ifndef PPR_PUSH_EARLY
+#define PPR_PUSH_EARLY 0
+#endif
+#ifndef PPR_PUSH_PIPE
+#define PPR_PUSH_PIPE 0
+#endif
+#ifndef PPR_PUSH_XCHG
+#define PPR_PUSH_XCHG 1
+#endif
 constexpr int U = PPR_PUSH_U;   // edges per lane per step
 constexpr int QW = 256;         // per-warp queue slice (entries)
 enum { M_OPT = 0, M_EAGER = 1, M_DUP = 2, M_VAN = 3, M_ASYNC = 4, M_SCAN = 5 };
@@ -217,7 +233,14 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     double* ru = Rp<PK>(a.g, sidx, u);
     double r = 0.0;
     bool push = false;
-    if (KIND == K_OPT || KIND == K_EAGER || KIND == K_SCAN) {
+    if (KIND == K_OPT && PPR_PUSH_XCHG) {
+        // Alg 4 lines 10 and 20-21 as one atomic: r_u = R(u), R(u) = 0.  Adds that
+        // reach u before the exchange are absorbed into r_u; adds
+        // after it start from 0, so u's next crossing re-enqueues it exactly once.
+        r = valid ? atom_exch_f64_pol(ru, 0.0, l2_keep()) : 0.0;
+        push = valid && r != 0.0;
+        if (push) red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
+    } else if (KIND == K_OPT || KIND == K_EAGER || KIND == K_SCAN) {
         r = valid ? ld_relaxed_f64(ru) : 0.0;  // Alg 4 line 10: the current R(u)
         // A queued vertex meets pushCond (it was enqueued on a crossing, and R(u)
         // only grows until its own self-update).  If the relaxed load returned
@@ -235,7 +258,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     // DESIGN.md K-PUSH) and P(u) += a r_u as a fire-and-forget reduction (one
     // entry per vertex per round, so no contention).
     double self_old = 0.0;
-    if (KIND == K_OPT && push) {
+    if (KIND == K_OPT && !PPR_PUSH_XCHG && push) {
         self_old = atomicAdd(ru, -r);
         red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
     }
@@ -269,7 +292,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     s.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
     s.sid[threadIdx.x] = sidx;
     __syncthreads();
-    if (a.trace && threadIdx.x == 0) c.t_pro += global_ns() - c.t_mark;
+    if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_pro += global_ns() - c.t_mark;
     if (threadIdx.x == 0) {
         c.edges += E;
         if (c.trace_edges && E) atomicAdd(c.trace_edges, (unsigned long long)E);
@@ -303,6 +326,79 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             }
         }
     } else {
+#if PPR_PUSH_PIPE
+    // software-pipelined walk: the pool entries (and owners) of the warp's next
+    // claim are loaded before the current claim's d_out loads and atomics, so a
+    // step costs the d_out -> atomic chain instead of pool -> d_out -> atomic
+    uint32_t cb = 0;
+    if (L == 0) cb = atomicAdd(&s.chunk, (unsigned)U);
+    cb = __shfl_sync(0xffffffffu, cb, 0);
+    uint32_t v[U];
+    int j[U];
+#pragma unroll
+    for (int k = 0; k < U; k++) {
+        const uint32_t e = (cb + k) * 32 + L;
+        j[k] = -1;
+        v[k] = 0;
+        if (e < E) {
+            j[k] = owner_of(s.scan, e, top);
+            v[k] = ld_u32_pol(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
+        }
+    }
+    while (cb * 32 < E) {
+        uint32_t cn = 0;
+        if (L == 0) cn = atomicAdd(&s.chunk, (unsigned)U);
+        cn = __shfl_sync(0xffffffffu, cn, 0);
+        uint32_t vn[U];
+        int jn[U];
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            const uint32_t e = (cn + k) * 32 + L;
+            jn[k] = -1;
+            vn[k] = 0;
+            if (e < E) {
+                jn[k] = owner_of(s.scan, e, top);
+                vn[k] = ld_u32_pol(&c.pool[s.off[jn[k]] + (e - s.scan[jn[k]])], pol_stream);
+            }
+        }
+        ensure_room(s, c, 32 * U);
+        uint32_t d[U];
+#pragma unroll
+        for (int k = 0; k < U; k++)
+            d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_pol(&a.g.dout[v[k]], pol_keep));
+        double incr[U], pre[U];
+        uint32_t sj[U];
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            if (j[k] >= 0) {
+                sj[k] = s.sid[j[k]];
+                incr[k] = __ddiv_rn(s.w[j[k]], (double)d[k]);
+                pre[k] = atom_add_pol(Rp<PK>(a.g, sj[k], v[k]), incr[k], pol_keep);
+            }
+        }
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            bool enq = false;
+            unsigned long long ev = 0;
+            if (j[k] >= 0) {
+                const double cur = __dadd_rn(pre[k], incr[k]);  // == the stored value (no FMA)
+                ev = ((unsigned long long)sj[k] << 32) | v[k];
+                if (KIND == K_OPT || KIND == K_DUP)
+                    enq = crossed<POS>(pre[k], cur, eps);   // Alg 4 line 16
+                else
+                    enq = push_cond<POS>(cur, eps) &&
+                          test_and_set(a.bitmap, (size_t)sj[k] * n + v[k]);  // UniqueEnqueue
+            }
+            warp_enqueue(s, c, enq, ev);
+        }
+        cb = cn;
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            v[k] = vn[k];
+            j[k] = jn[k];
+        }
+    }
+#else
 #if PPR_PUSH_DYN
     // warps claim U consecutive 32-edge chunks at a time from a shared counter,
     // so a warp whose atomics return late does not hold the tile's barrier
@@ -382,7 +478,10 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
         }
 #endif
     }
-    if (KIND == K_OPT) {  // re-enqueue on the result of the fused self-update
+#endif  // PPR_PUSH_PIPE
+    if (KIND == K_OPT && PPR_PUSH_XCHG) {
+        if (push) c.pushes++;
+    } else if (KIND == K_OPT) {  // re-enqueue on the result of the fused self-update
         bool re = false;
         if (push) {
             re = push_cond<POS>(__dadd_rn(self_old, -r), eps);
@@ -407,16 +506,33 @@ __device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a
     while (top * 2 < (int)T) top <<= 1;
     const uint64_t ntiles = (C + T - 1) / T;
     uint64_t t = blockIdx.x;
+#if PPR_PUSH_EARLY
+    // the claim of the CTA's next tile is issued before the current tile's work
+    // and read after it, so its round trip on the hot counter is hidden
+    const bool multi = ntiles > gridDim.x;
+    unsigned long long pending = 0;
+    if (multi && threadIdx.x == 0) pending = atomicAdd(tc, 1ull);
     while (t < ntiles) {
-        if (a.trace && threadIdx.x == 0) c.t_mark = global_ns();
         cta_tile<POS, KIND, PK>(s, c, a, Fin, C, t * T, T, top);
-        if (a.trace && threadIdx.x == 0) c.t_mark2 = global_ns();
+        if (!multi) break;
+        if (threadIdx.x == 0) s.next = pending + gridDim.x;
+        __syncthreads();
+        t = s.next;
+        __syncthreads();
+        if (t < ntiles && threadIdx.x == 0) pending = atomicAdd(tc, 1ull);
+    }
+    return;
+#endif
+    while (t < ntiles) {
+        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark = global_ns();
+        cta_tile<POS, KIND, PK>(s, c, a, Fin, C, t * T, T, top);
+        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark2 = global_ns();
         if (ntiles <= gridDim.x) break;  // every tile was assigned statically
         if (threadIdx.x == 0) s.next = atomicAdd(tc, 1ull) + gridDim.x;
         __syncthreads();
         t = s.next;
         __syncthreads();
-        if (a.trace && threadIdx.x == 0) c.t_claim += global_ns() - c.t_mark2;
+        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_claim += global_ns() - c.t_mark2;
     }
 }
 
@@ -594,7 +710,7 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
         c.Fout = a.F[(it + 1) & 1];
         c.cnt_out = &ctl->fcount[(it + 1) % 3].v;
         unsigned long long* tc = &ctl->tilectr[it % 3].v;
-        const unsigned long long t0 = a.trace ? global_ns() : 0;
+        const unsigned long long t0 = (kTimeSplit && a.trace) ? global_ns() : 0;
         if (MODE == M_OPT) {
             propagate_all<POS, K_OPT, PK>(s, c, a, Fin, C, tc);
         } else if (MODE == M_SCAN) {
@@ -615,11 +731,11 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
             grid_sync(ctl);
             session_eager_self<POS, PK>(s, c, a, Fin, C);
         }
-        const unsigned long long t1 = a.trace ? global_ns() : 0;
+        const unsigned long long t1 = (kTimeSplit && a.trace) ? global_ns() : 0;
         block_flush(s, c);
-        const unsigned long long t2 = a.trace ? global_ns() : 0;
+        const unsigned long long t2 = (kTimeSplit && a.trace) ? global_ns() : 0;
         grid_sync(ctl);
-        if (a.trace) {
+        if (kTimeSplit && a.trace) {
             const unsigned long long t3 = global_ns();
             c.t_work += t1 - t0;
             c.t_flush += t2 - t1;
@@ -663,7 +779,7 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
         a.trace[4ull * it] = ~0ull;  // end marker
         a.trace[4ull * it + 1] = global_ns();
     }
-    if (a.trace && threadIdx.x == 0) {  // per-CTA time split, summed over CTAs
+    if (kTimeSplit && a.trace && threadIdx.x == 0) {  // per-CTA time split, summed over CTAs
         atomicAdd(&a.trace[4ull * a.trace_cap + 0], c.t_work);
         atomicAdd(&a.trace[4ull * a.trace_cap + 1], c.t_flush);
         atomicAdd(&a.trace[4ull * a.trace_cap + 2], c.t_bar);

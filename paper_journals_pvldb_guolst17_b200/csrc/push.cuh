@@ -46,4 +46,18 @@ cudaError_t launch_push(int mode, const PushArgs& a, int num_sms, cudaStream_t s
 // PPR_MODE_SHARED: shared-adjacency multi-source push (push_ms.cu).
 cudaError_t launch_push_ms(const PushArgs& a, int num_sms, cudaStream_t st);
 
+// PPR_MODE_SORTAGG: host-driven Alg 3 rounds with sort-and-aggregate propagation
+// (push_sortagg.cu).  Synchronises the stream once or twice per round.
+struct SortAgg;  // scratch owned by the handle, grown on demand
+struct SortAggStats {
+    unsigned long long pushes = 0, edges = 0, max_frontier = 0;
+    unsigned iters[2] = {0, 0};
+    int noconv = 0;
+    unsigned active_pool = 0;  // in: which slab pool is active
+};
+cudaError_t sortagg_push(SortAgg** s, const PushArgs& a, uint64_t n_seed_v, cudaStream_t st,
+                         SortAggStats* out, uint32_t* launches);
+uint64_t sortagg_bytes(const SortAgg* s);
+void sortagg_free(SortAgg* s);
+
 }  // namespace ppr

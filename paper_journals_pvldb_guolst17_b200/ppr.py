@@ -20,10 +20,10 @@ LIB_PATH = os.path.join(_PKG, "libppr.so")
 PPR_OK, PPR_EINVAL, PPR_ERANGE, PPR_ENOENT, PPR_ENOMEM, PPR_ECUDA, PPR_EPOISONED, PPR_ENOCONV = \
     0, -1, -2, -3, -4, -5, -6, -7
 MEM_HOST, MEM_DEVICE = 0, 1
-MODE_OPT, MODE_EAGER, MODE_DUPDETECT, MODE_VANILLA, MODE_ASYNC, MODE_EAGER_SCAN, MODE_SHARED = \
-    0, 1, 2, 3, 4, 5, 6
+MODE_OPT, MODE_EAGER, MODE_DUPDETECT, MODE_VANILLA, MODE_ASYNC, MODE_EAGER_SCAN, MODE_SHARED, \
+    MODE_SORTAGG = 0, 1, 2, 3, 4, 5, 6, 7
 MODES = {"opt": MODE_OPT, "eager": MODE_EAGER, "dupdetect": MODE_DUPDETECT, "vanilla": MODE_VANILLA,
-         "async": MODE_ASYNC, "scan": MODE_EAGER_SCAN, "shared": MODE_SHARED}
+         "async": MODE_ASYNC, "scan": MODE_EAGER_SCAN, "shared": MODE_SHARED, "sortagg": MODE_SORTAGG}
 OPT_MODE, OPT_PUSH, OPT_MAX_ITERS, OPT_TIMING, OPT_FORCE_REBUILD = 1, 2, 3, 4, 5
 
 

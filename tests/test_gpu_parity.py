@@ -19,7 +19,7 @@ from tests import golden_figs as G
 
 pytestmark = pytest.mark.gpu
 
-MODES = ["opt", "eager", "dupdetect", "vanilla", "async", "scan", "shared"]
+MODES = ["opt", "eager", "dupdetect", "vanilla", "async", "scan", "shared", "sortagg"]
 
 
 def _fig_gpu(mode="vanilla", max_iters=0):
@@ -210,6 +210,70 @@ def test_shared_full_scan_push_matches_static():
         assert exact.terminated(R, 1e-8)
         Pstar = exact.ppr_power(cfg["n"], gs, gd, int(srcs[i]), 0.15)
         assert np.max(np.abs(P - Pstar)) <= 1e-8 * (1 + 1e-6)
+
+
+# ---------------------------------------------------------------- sort-and-aggregate (NEXT-4)
+
+def _tiny_static(mode, eps, sources=1, relabel=0):
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], sources)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=eps, mode=mode, relabel=relabel)
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, eps)
+    return st, cfg, srcs, h, o
+
+
+@pytest.mark.parametrize("eps,sources", [(1e-7, 1), (1e-9, 1), (1e-8, 3)])
+def test_sortagg_static_push_bit_exact_vs_alg3_oracle(eps, sources):
+    # PPR_MODE_SORTAGG applies each round's increments to R(v) in ascending-u
+    # order, exactly the oracle's Alg 3 emulation: same rounds,
+    # same pushes, and P, R equal bit for bit from P = 0, R = e_s
+    st, cfg, srcs, h, o = _tiny_static("sortagg", eps, sources)
+    o.push(oracle.JACOBI)
+    so, sg = o.stats(), h.create_stats
+    assert sg["pushes"] == so["pushes"] and sg["pushed_edges"] == so["pushed_edges"]
+    for i in range(sources):
+        P, R = h.query(i)
+        Po, Ro = o.query(i)
+        np.testing.assert_array_equal(R, Ro)
+        np.testing.assert_array_equal(P, Po)
+    if sources == 1:
+        assert sg["iters_pos"] == so["rounds_pos"] and sg["iters_neg"] == so["rounds_neg"]
+
+
+@pytest.mark.parametrize("rounds", [1, 4, 17])
+def test_sortagg_round_by_round_bit_exact(rounds):
+    # budgeted Alg 3 (max_iters rounds per phase) from P = 0, R = e_s
+    st, cfg, srcs, h, o = _tiny_static("sortagg", 1e-9)
+    h.reset()
+    h.set_option(ppr.OPT_MAX_ITERS, rounds)
+    stt = h.push()
+    assert stt["iters_pos"] == rounds
+    o2 = oracle.Oracle(cfg["n"], *st.window(), srcs, 0.15, 1e-9)
+    o2.set_state(0, np.zeros(cfg["n"]), np.eye(1, cfg["n"], int(srcs[0]))[0])
+    o2.push(oracle.JACOBI, max_steps=rounds)
+    P, R = h.query()
+    Po, Ro = o2.query()
+    np.testing.assert_array_equal(R, Ro)
+    np.testing.assert_array_equal(P, Po)
+
+
+def test_sortagg_bit_reproducible_across_runs():
+    # no atomics: two handles fed the same stream agree bit for bit after every
+    # batch (restore, store and push), also with degree-relabelled ids
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 2)
+    hs = [ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=1e-9, mode="sortagg", relabel=1)
+          for _ in range(2)]
+    for t in range(6):
+        b = st.next_batch()
+        for h in hs:
+            h.apply_batch(*b)
+        for i in range(2):
+            (P1, R1), (P2, R2) = hs[0].query(i), hs[1].query(i)
+            np.testing.assert_array_equal(P1, P2)
+            np.testing.assert_array_equal(R1, R2)
 
 
 def test_tiny_against_power_iteration():

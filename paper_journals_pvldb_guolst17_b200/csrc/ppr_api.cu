@@ -112,6 +112,7 @@ struct ppr_ctx {
     uint64_t buf_epoch = 0;                 // bumped whenever batch / pool buffers are reallocated
     unsigned long long* d_ring = nullptr;   // PPR_MODE_ASYNC ring queue (2*S*n slots, EMPTY)
     unsigned long long ring_cap = 0;
+    uint64_t hyb_thresh = 0;                // Opt: frontier size at which a phase finishes on the ring
     unsigned long long* d_trace = nullptr;  // PPR_TRACE=1: per-round trace of the push
     uint32_t trace_cap = 0;
     SortAgg* sa = nullptr;                  // PPR_MODE_SORTAGG scratch (grown on demand)
@@ -472,8 +473,20 @@ ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
         ppr_status rs = ensure_ring(h);
         if (rs != PPR_OK) return rs;
     }
+    if (h->mode == PPR_MODE_OPT && h->hyb_thresh && !h->d_ring && ensure_ring(h) != PPR_OK) {
+        h->hyb_thresh = 0;  // no room for the ring: rounds to the end
+        h->err.clear();
+    }
     a.ring = h->d_ring;
     a.ring_cap = h->ring_cap;
+    a.hyb_thresh = h->mode == PPR_MODE_OPT ? h->hyb_thresh : 0;
+    // dense graphs (>= 8 arcs per vertex) push on the ring from the start: rounds
+    // there only add barriers, no accumulation
+    {
+        const char* ha = getenv("PPR_HYBRID_ALL");
+        const bool dense = (double)h->m >= 8.0 * (double)h->n;
+        a.hyb_all = (a.hyb_thresh && (ha ? atoi(ha) > 0 : dense)) ? 1 : 0;
+    }
     cudaError_t e = launch_push(h->mode, a, h->num_sms, h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, "push launch");
     ++*launches;
@@ -634,6 +647,12 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     cudaEventCreateWithFlags(&h->ev_join, cudaEventDisableTiming);
     h->npasses = key_shifts(ceil_log2(h->n), h->shifts);
     if (getenv("PPR_GRAPHS") && !strcmp(getenv("PPR_GRAPHS"), "0")) h->graphs = false;
+    {   // hybrid tail: PPR_HYBRID=<entries>, 0 = off; the ring
+        // costs 16 B per (source, vertex), so it is only used up to 2^27 of them
+        const char* hy = getenv("PPR_HYBRID");
+        const long long t = hy ? atoll(hy) : 16384;
+        h->hyb_thresh = (t > 0 && (uint64_t)h->S * h->n <= (1ull << 27)) ? (uint64_t)t : 0;
+    }
     if (getenv("PPR_TRACE") && atoi(getenv("PPR_TRACE")) > 0) {
         h->trace_cap = 4096;
         dalloc(h, &h->d_trace, 4ull * h->trace_cap + 8);

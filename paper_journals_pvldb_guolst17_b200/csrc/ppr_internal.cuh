@@ -71,6 +71,7 @@ struct __align__(128) HotU32 {
 struct DevCtl {
     HotU64 fcount[3];   // frontier counters, triple-buffered by round (push.cu)
     HotU64 tilectr[3];  // tile claims, triple-buffered by round
+    HotU64 hyb[3];      // hybrid tail ring: head, tail, done (push.cu)
     HotU32 bar_count;   // grid barrier arrivals
     HotU32 bar_gen;     // grid barrier generation
     DevStats st;

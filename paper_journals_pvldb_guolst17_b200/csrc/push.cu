@@ -61,12 +61,6 @@ constexpr int NW = PT / 32;     // warps per CTA
 #define PPR_PUSH_TIMESPLIT 0
 #endif
 constexpr bool kTimeSplit = PPR_PUSH_TIMESPLIT;
-#ifndef PPR_PUSH_EARLY
-#define PPR_PUSH_EARLY 0
-#endif
-#ifndef PPR_PUSH_PIPE
-#define PPR_PUSH_PIPE 0
-#endif
 #ifndef PPR_PUSH_XCHG
 #define PPR_PUSH_XCHG 1
 #endif
@@ -326,79 +320,6 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             }
         }
     } else {
-#if PPR_PUSH_PIPE
-    // software-pipelined walk: the pool entries (and owners) of the warp's next
-    // claim are loaded before the current claim's d_out loads and atomics, so a
-    // step costs the d_out -> atomic chain instead of pool -> d_out -> atomic
-    uint32_t cb = 0;
-    if (L == 0) cb = atomicAdd(&s.chunk, (unsigned)U);
-    cb = __shfl_sync(0xffffffffu, cb, 0);
-    uint32_t v[U];
-    int j[U];
-#pragma unroll
-    for (int k = 0; k < U; k++) {
-        const uint32_t e = (cb + k) * 32 + L;
-        j[k] = -1;
-        v[k] = 0;
-        if (e < E) {
-            j[k] = owner_of(s.scan, e, top);
-            v[k] = ld_u32_pol(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
-        }
-    }
-    while (cb * 32 < E) {
-        uint32_t cn = 0;
-        if (L == 0) cn = atomicAdd(&s.chunk, (unsigned)U);
-        cn = __shfl_sync(0xffffffffu, cn, 0);
-        uint32_t vn[U];
-        int jn[U];
-#pragma unroll
-        for (int k = 0; k < U; k++) {
-            const uint32_t e = (cn + k) * 32 + L;
-            jn[k] = -1;
-            vn[k] = 0;
-            if (e < E) {
-                jn[k] = owner_of(s.scan, e, top);
-                vn[k] = ld_u32_pol(&c.pool[s.off[jn[k]] + (e - s.scan[jn[k]])], pol_stream);
-            }
-        }
-        ensure_room(s, c, 32 * U);
-        uint32_t d[U];
-#pragma unroll
-        for (int k = 0; k < U; k++)
-            d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_pol(&a.g.dout[v[k]], pol_keep));
-        double incr[U], pre[U];
-        uint32_t sj[U];
-#pragma unroll
-        for (int k = 0; k < U; k++) {
-            if (j[k] >= 0) {
-                sj[k] = s.sid[j[k]];
-                incr[k] = __ddiv_rn(s.w[j[k]], (double)d[k]);
-                pre[k] = atom_add_pol(Rp<PK>(a.g, sj[k], v[k]), incr[k], pol_keep);
-            }
-        }
-#pragma unroll
-        for (int k = 0; k < U; k++) {
-            bool enq = false;
-            unsigned long long ev = 0;
-            if (j[k] >= 0) {
-                const double cur = __dadd_rn(pre[k], incr[k]);  // == the stored value (no FMA)
-                ev = ((unsigned long long)sj[k] << 32) | v[k];
-                if (KIND == K_OPT || KIND == K_DUP)
-                    enq = crossed<POS>(pre[k], cur, eps);   // Alg 4 line 16
-                else
-                    enq = push_cond<POS>(cur, eps) &&
-                          test_and_set(a.bitmap, (size_t)sj[k] * n + v[k]);  // UniqueEnqueue
-            }
-            warp_enqueue(s, c, enq, ev);
-        }
-        cb = cn;
-#pragma unroll
-        for (int k = 0; k < U; k++) {
-            v[k] = vn[k];
-            j[k] = jn[k];
-        }
-    }
-#else
 #if PPR_PUSH_DYN
     // warps claim U consecutive 32-edge chunks at a time from a shared counter,
     // so a warp whose atomics return late does not hold the tile's barrier
@@ -478,7 +399,6 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
         }
 #endif
     }
-#endif  // PPR_PUSH_PIPE
     if (KIND == K_OPT && PPR_PUSH_XCHG) {
         if (push) c.pushes++;
     } else if (KIND == K_OPT) {  // re-enqueue on the result of the fused self-update
@@ -506,23 +426,6 @@ __device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a
     while (top * 2 < (int)T) top <<= 1;
     const uint64_t ntiles = (C + T - 1) / T;
     uint64_t t = blockIdx.x;
-#if PPR_PUSH_EARLY
-    // the claim of the CTA's next tile is issued before the current tile's work
-    // and read after it, so its round trip on the hot counter is hidden
-    const bool multi = ntiles > gridDim.x;
-    unsigned long long pending = 0;
-    if (multi && threadIdx.x == 0) pending = atomicAdd(tc, 1ull);
-    while (t < ntiles) {
-        cta_tile<POS, KIND, PK>(s, c, a, Fin, C, t * T, T, top);
-        if (!multi) break;
-        if (threadIdx.x == 0) s.next = pending + gridDim.x;
-        __syncthreads();
-        t = s.next;
-        __syncthreads();
-        if (t < ntiles && threadIdx.x == 0) pending = atomicAdd(tc, 1ull);
-    }
-    return;
-#endif
     while (t < ntiles) {
         if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark = global_ns();
         cta_tile<POS, KIND, PK>(s, c, a, Fin, C, t * T, T, top);
@@ -672,6 +575,38 @@ __device__ __forceinline__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
     }
 }
 
+// ---------------------------------------------------------------- hybrid tail
+//
+// Opt mode, PushArgs::hyb_thresh > 0: once a phase's frontier has shrunk to
+// at most hyb_thresh entries, its remaining rounds are latency-bound (a few
+// microseconds of dependent loads and atomics plus a grid barrier per round,
+// for a few thousand pushes), so the rest of the phase runs on the
+// asynchronous ring schedule instead (the same operations without round
+// barriers; any push order is valid, Lemma 1; DESIGN.md K-ASYNC).
+template <bool POS, bool PK>
+__device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, unsigned long long* head,
+                                           unsigned long long* tail, unsigned long long* done);
+
+template <bool POS, bool PK>
+__device__ __forceinline__ void hybrid_tail(Smem& s, Ctx& c, const PushArgs& a,
+                                            const unsigned long long* Fin, uint64_t C) {
+    DevCtl* ctl = a.ctl;
+    unsigned long long* head = &ctl->hyb[0].v;
+    unsigned long long* tail = &ctl->hyb[1].v;
+    unsigned long long* done = &ctl->hyb[2].v;
+    for (uint64_t i = (uint64_t)blockIdx.x * PT + threadIdx.x; i < C; i += (uint64_t)gridDim.x * PT)
+        __stcg(&a.ring[i], __ldcg(&Fin[i]));  // ring slots are EMPTY between uses
+    if (blockIdx.x == 0 && threadIdx.x == 0) *tail = C;
+    grid_sync(ctl);
+    c.Fout = a.ring;
+    c.cnt_out = tail;
+    c.ring_cap = a.ring_cap;
+    async_loop<POS, PK>(s, c, a, head, tail, done);
+    c.ring_cap = 0;
+    grid_sync(ctl);
+    if (blockIdx.x == 0 && threadIdx.x == 0) *head = *tail = *done = 0;
+}
+
 // ---------------------------------------------------------------- phase driver
 
 template <int MODE, bool POS, bool PK>
@@ -685,7 +620,7 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
     block_flush(s, c);
     grid_sync(ctl);
     uint32_t pit = 0;
-    uint64_t C = 0;
+    uint64_t C = 0, Cprev = ~0ull;
     while (true) {
         // one load per CTA (grid_sync ended with __syncthreads)
         if (threadIdx.x == 0) s.cround = *(volatile unsigned long long*)&ctl->fcount[it % 3].v;
@@ -707,6 +642,15 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
         }
         if (C == 0 || (a.max_iters && pit >= a.max_iters) || pit >= a.iter_cap) break;
         const unsigned long long* Fin = a.F[it & 1];
+        // the ring takes over: for the whole phase on dense graphs (hyb_all), else
+        // once the frontier is past its peak and at most hyb_thresh entries
+        if (MODE == M_OPT && a.ring && !a.max_iters &&
+            (a.hyb_all || (pit > 0 && C <= a.hyb_thresh && C <= Cprev))) {
+            hybrid_tail<POS, PK>(s, c, a, Fin, C);  // the phase ends on the ring
+            it++;
+            C = 0;
+            break;
+        }
         c.Fout = a.F[(it + 1) & 1];
         c.cnt_out = &ctl->fcount[(it + 1) % 3].v;
         unsigned long long* tc = &ctl->tilectr[it % 3].v;
@@ -743,6 +687,7 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
         }
         it++;
         pit++;
+        Cprev = C;
     }
     // a frontier left by max_iters keeps its UniqueEnqueue bits: drop them
     if ((MODE == M_VAN || MODE == M_EAGER) && C > 0) clear_frontier_bits(c, a, a.F[it & 1], C);
@@ -842,18 +787,12 @@ inline cudaError_t coop_launch(const void* fn, int grid, const PushArgs& a, cuda
 // entry's children are added to tail before the entry is added to done, so
 // reading done == tail (done first) means no entry is queued or in progress.
 
+// The ring loop: CTAs claim chunks of queued entries and process each chunk
+// as a tile until done == tail.  Entry: the ring holds the seeds, tail = their
+// count, head = done = 0, c.Fout/c.cnt_out/c.ring_cap point at the ring.
 template <bool POS, bool PK>
-__device__ __forceinline__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
-    DevCtl* ctl = a.ctl;
-    unsigned long long* head = &ctl->tilectr[0].v;
-    unsigned long long* tail = &ctl->fcount[0].v;
-    unsigned long long* done = &ctl->fcount[1].v;
-    c.Fout = a.ring;
-    c.cnt_out = tail;
-    c.ring_cap = a.ring_cap;
-    seed_phase<POS, PK>(s, c, a);
-    block_flush(s, c);
-    grid_sync(ctl);
+__device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, unsigned long long* head,
+                                           unsigned long long* tail, unsigned long long* done) {
     __shared__ unsigned long long s_h, s_k;
     __shared__ int s_flag;
     unsigned long long debt_lo = 0, debt_hi = 0;  // thread 0: claimed, not yet served
@@ -912,6 +851,21 @@ __device__ __forceinline__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) 
         block_flush(s, c);  // this tile's children reach `tail` ...
         if (threadIdx.x == 0) atomicAdd(done, (unsigned long long)k);  // ... before it counts as done
     }
+}
+
+template <bool POS, bool PK>
+__device__ __forceinline__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
+    DevCtl* ctl = a.ctl;
+    unsigned long long* head = &ctl->tilectr[0].v;
+    unsigned long long* tail = &ctl->fcount[0].v;
+    unsigned long long* done = &ctl->fcount[1].v;
+    c.Fout = a.ring;
+    c.cnt_out = tail;
+    c.ring_cap = a.ring_cap;
+    seed_phase<POS, PK>(s, c, a);
+    block_flush(s, c);
+    grid_sync(ctl);
+    async_loop<POS, PK>(s, c, a, head, tail, done);
     grid_sync(ctl);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         *head = 0;

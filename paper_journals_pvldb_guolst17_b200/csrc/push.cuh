@@ -36,6 +36,8 @@ struct PushArgs {
     uint32_t iter_cap;         // safety cap -> KERR_NOCONV
     unsigned long long* ring;  // async mode: ring queue of ring_cap slots, all EMPTY between calls
     unsigned long long ring_cap;
+    int hyb_all;               // Opt: every phase runs on the ring from its seeds (dense graphs)
+    uint64_t hyb_thresh;       // Opt: a phase whose frontier is <= this many entries finishes on the ring (0: off)
     unsigned long long* trace; // optional: 4 words per round {C | phase<<63, t_ns, edges, -}
     uint32_t trace_cap;        // rounds the trace buffer holds
 };

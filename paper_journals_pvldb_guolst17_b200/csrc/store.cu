@@ -19,6 +19,9 @@
 // insertion and a deletion of the same arc in one batch cancel exactly.
 #include "block_scan.cuh"
 #include "primitives.cuh"
+#include <algorithm>
+#include <cstdlib>
+
 #include "store.cuh"
 
 namespace ppr {
@@ -598,13 +601,27 @@ __global__ void k_degree_keys(const uint32_t* __restrict__ deg, uint32_t n, uint
     }
 }
 
+// spread = k > 0 (default 1; PPR_RELABEL_SPREAD): inside every full block of
+// 16 L ranks (L = 16^k lines of 16 residuals) rank i goes to line i % L, slot
+// i / L, so consecutive (equally hot) ranks land on different 128-byte residual
+// lines -- and L2 slices -- while the block's footprint stays L lines (measured:
+// Orkut-shaped relabelled push 29.8 -> 27.9 ms, LJ 3.26 -> 3.23 ms; DESIGN.md
+// "Relabelling")
 __global__ void k_perm_from_sorted(const uint64_t* __restrict__ keys, uint32_t n,
-                                   uint32_t* __restrict__ perm, uint32_t* __restrict__ inv) {
+                                   uint32_t* __restrict__ perm, uint32_t* __restrict__ inv, int spread) {
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
          i += (uint64_t)gridDim.x * blockDim.x) {
         const uint32_t v = (uint32_t)keys[i];
-        inv[i] = v;
-        perm[v] = (uint32_t)i;
+        uint32_t id = (uint32_t)i;
+        if (spread) {  // block of 16 * L ranks: rank i -> line i % L, slot i / L
+            const uint32_t L = 16u << (4 * (spread - 1)), B = 16u * L;
+            if ((id / B + 1) * (uint64_t)B <= n) {
+                const uint32_t j = id % B;
+                id = id - j + (j % L) * 16u + j / L;
+            }
+        }
+        inv[id] = v;
+        perm[v] = id;
     }
 }
 
@@ -784,7 +801,9 @@ void launch_relabel(const uint32_t* src, const uint32_t* dst, uint64_t m, int un
     for (int s = 0; s < lg; s += 8) shifts[np++] = s;
     for (int s = 32; s < 64; s += 8) shifts[np++] = s;
     const int w = radix_sort_pairs(k0, v0, k1, v1, n, shifts, np, hist, st, launches);
-    k_perm_from_sorted<<<grid_for(n, 256), 256, 0, st>>>(w ? k1 : k0, n, perm, inv);
+    const char* sp = getenv("PPR_RELABEL_SPREAD");
+    const int spread = sp ? std::max(0, std::min(3, atoi(sp))) : 1;
+    k_perm_from_sorted<<<grid_for(n, 256), 256, 0, st>>>(w ? k1 : k0, n, perm, inv, spread);
     *launches += 3;
 }
 

@@ -136,6 +136,16 @@ def test_tiny_config_all_modes_track_oracle(mode):
     _run_stream("tiny", mode, slides=12)
 
 
+@pytest.mark.parametrize("hyb,hyb_all", [("0", "0"), ("16384", "0"), ("16384", "1"), ("64", "0")])
+def test_opt_schedules_track_oracle(monkeypatch, hyb, hyb_all):
+    # Opt rounds only / rounds with the ring tail / ring from the seeds (DESIGN.md
+    # "Hybrid tail"): every schedule meets the same gates
+    monkeypatch.setenv("PPR_HYBRID", hyb)
+    monkeypatch.setenv("PPR_HYBRID_ALL", hyb_all)
+    _run_stream("tiny", "opt", slides=6)
+    _run_stream("tiny", "opt", slides=3, sources=3)
+
+
 @pytest.mark.parametrize("mode", ["opt", "scan", "vanilla"])
 def test_tiny_config_degree_relabelled(mode):
     # internal degree-ordered ids: every id at the boundary must stay external

@@ -164,6 +164,9 @@ __device__ __forceinline__ void st_release_u32(unsigned int* p, unsigned int v) 
 }
 
 // Sense-free generation barrier over all CTAs of a cooperative launch.
+#ifndef PPR_BAR_SLEEP
+#define PPR_BAR_SLEEP 32
+#endif
 __device__ __forceinline__ void grid_sync(DevCtl* ctl) {
     __syncthreads();
     if (threadIdx.x == 0) {
@@ -175,7 +178,8 @@ __device__ __forceinline__ void grid_sync(DevCtl* ctl) {
             __threadfence();
             st_release_u32(&ctl->bar_gen.v, gen + 1u);
         } else {
-            while (ld_acquire_u32(&ctl->bar_gen.v) == gen) __nanosleep(32);
+            while (ld_acquire_u32(&ctl->bar_gen.v) == gen)
+                if (PPR_BAR_SLEEP) __nanosleep(PPR_BAR_SLEEP);
         }
         __threadfence();
     }

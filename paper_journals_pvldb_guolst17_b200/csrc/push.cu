@@ -65,7 +65,10 @@ constexpr bool kTimeSplit = PPR_PUSH_TIMESPLIT;
 #define PPR_PUSH_XCHG 1
 #endif
 constexpr int U = PPR_PUSH_U;   // edges per lane per step
-constexpr int QW = 256;         // per-warp queue slice (entries)
+#ifndef PPR_PUSH_QW
+#define PPR_PUSH_QW 256
+#endif
+constexpr int QW = PPR_PUSH_QW; // per-warp queue slice (entries)
 enum { M_OPT = 0, M_EAGER = 1, M_DUP = 2, M_VAN = 3, M_ASYNC = 4, M_SCAN = 5 };
 // how a warp tile gets r and decides enqueues
 enum { K_OPT = 0, K_EAGER = 1, K_DUP = 2, K_VAN = 3, K_SCAN = 4 };

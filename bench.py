@@ -61,6 +61,9 @@ def parse():
     p.add_argument("--seed", type=int, default=42)
     p.add_argument("--band", type=int, default=None,
                    help="sources drawn from the top-BAND out-degree vertices (default: the config's 1000)")
+    p.add_argument("--shard", default=None,
+                   help="R/G: run only rank R's source shard of a G-GPU run on this one GPU "
+                        "(per-rank load of a multi-GPU run; scaling projection)")
     p.add_argument("--no-cpu-baseline", action="store_true")
     p.add_argument("--cpu-budget-s", type=float, default=30.0)
     p.add_argument("--ref-budget-s", type=float, default=150.0)
@@ -238,7 +241,9 @@ def config_block(args, cfg, eps, S):
             "rmat_abc": list(cfg["abc"]), "mode": args.mode,
             "internal_ids": {1: "G0 out-degree order", 0: "external", -1: "auto (degree order iff R+d_out > 48 MB)"}[args.relabel],
             "l2": ("persisting lines reset + flushed between steps (512 MiB write)"
-                   if not args.no_flush else "not flushed")}
+                   if not args.no_flush else "not flushed"),
+            **({"shard": f"rank {args.shard} of the sources (one GPU's load of a multi-GPU run)"}
+               if getattr(args, "shard", None) else {})}
 
 
 # ---------------------------------------------------------------- our arm
@@ -319,7 +324,12 @@ def run_ours(args):
     deg = np.bincount(win_np[0], minlength=cfg["n"])
     if und:
         deg = deg + np.bincount(win_np[1], minlength=cfg["n"])
-    my_srcs = D.partition_sources(srcs_all, deg, ws, rank)
+    if args.shard:
+        sr, sg = (int(x) for x in args.shard.split("/"))
+        assert ws == 1 and 0 <= sr < sg, "--shard R/G emulates one rank of G on a single process"
+        my_srcs = D.partition_sources(srcs_all, deg, sg, sr)
+    else:
+        my_srcs = D.partition_sources(srcs_all, deg, ws, rank)
     if args.mode == "auto":  # measured: Opt best single-source, SHARED for several sources per rank
         args.mode = "opt" if len(my_srcs) == 1 else "shared"
 

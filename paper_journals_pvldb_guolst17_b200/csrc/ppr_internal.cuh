@@ -225,6 +225,31 @@ __device__ __forceinline__ uint32_t ld_u32_pol(const uint32_t* a, unsigned long 
     asm volatile("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
     return r;
 }
+// the push's two per-edge loads: the pool entry is streamed (read once per
+// walk: PPR_L1_POOL_NA=1 keeps it out of L1), d_out(v) is re-read for every
+// pushed in-arc of v (PPR_L1_DOUT_EL=1 asks L1 to keep it)
+#ifndef PPR_L1_POOL_NA
+#define PPR_L1_POOL_NA 0
+#endif
+#ifndef PPR_L1_DOUT_EL
+#define PPR_L1_DOUT_EL 0
+#endif
+__device__ __forceinline__ uint32_t ld_pool(const uint32_t* a, unsigned long long pol) {
+    uint32_t r;
+    if (PPR_L1_POOL_NA)
+        asm volatile("ld.global.nc.L1::no_allocate.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
+    else
+        asm volatile("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
+    return r;
+}
+__device__ __forceinline__ uint32_t ld_dout(const uint32_t* a, unsigned long long pol) {
+    uint32_t r;
+    if (PPR_L1_DOUT_EL)
+        asm volatile("ld.global.nc.L1::evict_last.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
+    else
+        asm volatile("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
+    return r;
+}
 __device__ __forceinline__ ulonglong2 ld_u64x2_pol(const void* a, unsigned long long pol) {
     ulonglong2 r;
     asm volatile("ld.global.nc.L2::cache_hint.v2.u64 {%0, %1}, [%2], %3;"

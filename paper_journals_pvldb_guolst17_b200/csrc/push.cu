@@ -307,12 +307,12 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
                 v[k] = 0;
                 if (e < E) {
                     j[k] = owner_of(s.scan, e, top);
-                    v[k] = ld_u32_pol(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
+                    v[k] = ld_pool(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
                 }
             }
 #pragma unroll
             for (int k = 0; k < U; k++)
-                d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_pol(&a.g.dout[v[k]], pol_keep));
+                d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_dout(&a.g.dout[v[k]], pol_keep));
 #pragma unroll
             for (int k = 0; k < U; k++) {
                 if (j[k] >= 0) {
@@ -346,13 +346,13 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             v[k] = 0;
             if (e < E) {
                 j[k] = owner_of(s.scan, e, top);
-                v[k] = ld_u32_pol(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
+                v[k] = ld_pool(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
             }
         }
         uint32_t d[U];
 #pragma unroll
         for (int k = 0; k < U; k++)
-            d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_pol(&a.g.dout[v[k]], pol_keep));
+            d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_dout(&a.g.dout[v[k]], pol_keep));
 #if PPR_PUSH_OVERLAP
         // all U atomics are issued before any result is consumed, so the U
         // chains overlap (the enqueues below synchronise the warp)

@@ -140,37 +140,70 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
     const uint32_t S = a.g.S;
     const double eps = a.g.eps, alpha = a.g.alpha;
     const unsigned long long pol_keep = l2_keep(), pol_stream = l2_stream();
-    // Phase A: one warp per entry -- eager row read, push mask, self-update
-    for (uint32_t j = w; j < T; j += NW) {
-        const uint64_t idx = base + j;
-        const bool ve = idx < C;  // warp-uniform
-        const unsigned long long ent = ve ? __ldcg(&Fin[idx]) : 0ull;
-        const uint32_t g = (uint32_t)(ent >> 32), u = (uint32_t)ent;
-        ulonglong2 sl = make_ulonglong2(0, 0);
-        if (ve && L == 0) sl = ld_u64x2_pol(&a.g.slab[u], pol_stream);  // Slab {off, len|cap}
-        const uint32_t sidx = g * 32 + L;
-        const bool lok = ve && sidx < S;
-        double* ru = a.g.R + (size_t)u * S + sidx;
-        const double r = lok ? ld_relaxed_f64(ru) : 0.0;
-        const bool p = lok && push_cond<POS>(r, eps);
-        const unsigned mask = __ballot_sync(0xffffffffu, p);
-        if (p) {
-            red_add_pol(ru, -r, pol_keep);
-            red_add_pol(a.g.P + (size_t)u * S + sidx, __dmul_rn(alpha, r), pol_stream);
+    // Phase A: one warp per entry -- eager row read, push mask, self-update.
+    // A warp's entries are j = w + NW*i, i < PA (at most MT/NW): lane i loads
+    // entry i and its slab descriptor, then the warp issues all PA row reads
+    // before consuming any, so the entries' dependent loads overlap instead of
+    // running one chain per entry.
+    constexpr int PA = MT / NW;
+    static_assert(PA <= 32, "one lane per entry of the warp");
+    unsigned long long myent = 0;
+    ulonglong2 mysl = make_ulonglong2(0, 0);
+    {
+        const uint32_t j = w + NW * L;
+        if (L < (unsigned)PA && j < T && base + j < C) {
+            myent = __ldcg(&Fin[base + j]);
+            mysl = ld_u64x2_pol(&a.g.slab[(uint32_t)myent], pol_stream);  // Slab {off, len|cap}
         }
-        s.w[j][L] = p ? __dmul_rn(1.0 - alpha, r) : 0.0;
-        if (L == 0) {
-            const uint32_t len = mask ? (uint32_t)sl.y : 0u;
-            s.len[j] = len;
-            s.off[j] = sl.x;
-            s.grp[j] = g;
-            if (mask) {
-                mark(a.bitmap, (unsigned long long)u * SG + g);  // u's row changed
-                const unsigned k = __popc(mask);
-                c.pushes += k;
-                c.edges += (unsigned long long)k * len;
-                c.walks += len;
+    }
+    unsigned mymask = 0;
+    constexpr int PB = 4;  // row reads in flight per batch (registers)
+#pragma unroll
+    for (int i0 = 0; i0 < PA; i0 += PB) {
+        if (w + NW * i0 >= T) break;  // warp-uniform
+        double r[PB];
+#pragma unroll
+        for (int q = 0; q < PB; q++) {
+            const int i = i0 + q;
+            const unsigned long long ent = __shfl_sync(0xffffffffu, myent, i);
+            const uint32_t j = w + NW * i;
+            const uint32_t sidx = (uint32_t)(ent >> 32) * 32 + L;
+            const bool lok = j < T && base + j < C && sidx < S;
+            r[q] = lok ? ld_relaxed_f64(a.g.R + (size_t)(uint32_t)ent * S + sidx) : 0.0;
+        }
+#pragma unroll
+        for (int q = 0; q < PB; q++) {
+            const int i = i0 + q;
+            const uint32_t j = w + NW * i;
+            if (j >= T) break;  // warp-uniform
+            const unsigned long long ent = __shfl_sync(0xffffffffu, myent, i);
+            const uint32_t g = (uint32_t)(ent >> 32), u = (uint32_t)ent;
+            const uint32_t sidx = g * 32 + L;
+            const bool p = base + j < C && sidx < S && push_cond<POS>(r[q], eps);
+            const unsigned mask = __ballot_sync(0xffffffffu, p);
+            if (p) {
+                red_add_pol(a.g.R + (size_t)u * S + sidx, -r[q], pol_keep);
+                red_add_pol(a.g.P + (size_t)u * S + sidx, __dmul_rn(alpha, r[q]), pol_stream);
             }
+            s.w[j][L] = p ? __dmul_rn(1.0 - alpha, r[q]) : 0.0;
+            if (L == (unsigned)i) mymask = mask;
+            if (L == 0 && mask) {  // u's row changed (one mark per entry: no test needed)
+                const unsigned long long bit = (unsigned long long)u * SG + g;
+                atomicOr(&a.bitmap[bit >> 5], 1u << (bit & 31u));
+            }
+        }
+    }
+    if (L < (unsigned)PA && w + NW * L < T) {  // lane i publishes entry i
+        const uint32_t j = w + NW * L;
+        const uint32_t len = mymask ? (uint32_t)mysl.y : 0u;
+        s.len[j] = len;
+        s.off[j] = mysl.x;
+        s.grp[j] = (uint32_t)(myent >> 32);
+        if (mymask) {
+            const unsigned k = __popc(mymask);
+            c.pushes += k;
+            c.edges += (unsigned long long)k * len;
+            c.walks += len;
         }
     }
     __syncthreads();
@@ -210,8 +243,8 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
         uint32_t v = 0, d = 1;
         if (ok) {
             j = owner_of(s.scan, e, top);
-            v = ld_u32_pol(&c.pool[s.off[j] + (e - s.scan[j])], pol_stream);
-            d = ld_u32_pol(&a.g.dout[v], pol_keep);
+            v = ld_pool(&c.pool[s.off[j] + (e - s.scan[j])], pol_stream);
+            d = ld_dout(&a.g.dout[v], pol_keep);
             mark(a.bitmap, (unsigned long long)v * SG + s.grp[j]);
         }
         const double rd = __drcp_rn((double)d);

@@ -41,8 +41,15 @@ namespace {
 
 constexpr int PT = PUSH_THREADS;
 constexpr int NW = PT / 32;
-constexpr int MT = 64;    // frontier entries per CTA tile
-constexpr int QW = 256;   // per-warp queue slice (entries)
+#ifndef PPR_MS_MT
+#define PPR_MS_MT 64
+#endif
+constexpr int MT = PPR_MS_MT;  // frontier entries per CTA tile (a multiple of 32)
+static_assert(MT % 32 == 0, "MT");
+#ifndef PPR_MS_QW
+#define PPR_MS_QW 256
+#endif
+constexpr int QW = PPR_MS_QW;  // per-warp queue slice (entries)
 
 struct MsSmem {
     double w[MT][32];                 // (1-a) r of every lane of every entry (0: lane idle)
@@ -207,21 +214,29 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
         }
     }
     __syncthreads();
-    // exclusive scan of the T walk lengths (warp 0, two entries per lane)
+    // exclusive scan of the T walk lengths (warp 0, MT/32 consecutive entries per lane)
     if (w == 0) {
-        const uint32_t a0 = 2 * L < T ? s.len[2 * L] : 0u;
-        const uint32_t a1 = 2 * L + 1 < T ? s.len[2 * L + 1] : 0u;
-        uint32_t inc = a0 + a1;
+        constexpr int EPL = MT / 32;
+        uint32_t x[EPL];
+        uint32_t sum = 0;
+#pragma unroll
+        for (int q = 0; q < EPL; q++) {
+            x[q] = EPL * L + q < T ? s.len[EPL * L + q] : 0u;
+            sum += x[q];
+        }
+        uint32_t inc = sum;
 #pragma unroll
         for (int o = 1; o < 32; o <<= 1) {
             const uint32_t y = __shfl_up_sync(0xffffffffu, inc, o);
             if (L >= (unsigned)o) inc += y;
         }
-        const uint32_t ex = inc - a0 - a1;
-        s.scan[2 * L] = 2 * L < T ? ex : 0xFFFFFFFFu;
-        s.scan[2 * L + 1] = 2 * L + 1 < T ? ex + a0 : 0xFFFFFFFFu;
-        s.scan[2 * L + MT] = 0xFFFFFFFFu;
-        s.scan[2 * L + 1 + MT] = 0xFFFFFFFFu;
+        uint32_t ex = inc - sum;
+#pragma unroll
+        for (int q = 0; q < EPL; q++) {
+            s.scan[EPL * L + q] = EPL * L + q < T ? ex : 0xFFFFFFFFu;
+            s.scan[EPL * L + q + MT] = 0xFFFFFFFFu;
+            ex += x[q];
+        }
         if (L == 31) {
             s.E = inc;
             s.chunk = 0;

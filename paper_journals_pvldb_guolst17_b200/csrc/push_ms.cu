@@ -44,6 +44,12 @@ constexpr int NW = PT / 32;
 #ifndef PPR_MS_MT
 #define PPR_MS_MT 64
 #endif
+#ifndef PPR_MS_CLAIM_AHEAD
+#define PPR_MS_CLAIM_AHEAD 1
+#endif
+#ifndef PPR_MS_WSCAN
+#define PPR_MS_WSCAN 1
+#endif
 constexpr int MT = PPR_MS_MT;  // frontier entries per CTA tile (a multiple of 32)
 static_assert(MT % 32 == 0, "MT");
 #ifndef PPR_MS_QW
@@ -64,6 +70,10 @@ struct MsSmem {
     unsigned long long cround;
     unsigned int chunk;
     uint32_t E;
+#if PPR_MS_WSCAN
+    uint32_t wscan[NW][2 * MT];       // every warp's own copy of the prefix (no scan barrier)
+    unsigned int chunk2[2];           // chunk counters of even / odd tiles
+#endif
 };
 
 struct MsCtx {
@@ -74,6 +84,7 @@ struct MsCtx {
     unsigned long long pushes;     // (source, vertex) self-updates
     unsigned long long edges;      // (source, arc) propagations
     unsigned long long walks;      // (group, arc) walks
+    uint32_t tiles;                // tiles processed by this CTA (chunk-counter parity)
 };
 
 __device__ __forceinline__ unsigned lane() { return threadIdx.x & 31u; }
@@ -214,8 +225,19 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
         }
     }
     __syncthreads();
-    // exclusive scan of the T walk lengths (warp 0, MT/32 consecutive entries per lane)
+    // exclusive scan of the T walk lengths (MT/32 consecutive entries per lane);
+    // with PPR_MS_WSCAN every warp computes it into its own copy, so the walk
+    // starts without a second CTA barrier (the chunk counter of this tile's
+    // parity was reset during the previous tile)
+#if PPR_MS_WSCAN
+    uint32_t Ew = 0;  // the tile's walk length, from every warp's own scan
+    const uint32_t par = c.tiles & 1u;
+    uint32_t* scan = s.wscan[w];
+    if (true) {
+#else
+    uint32_t* scan = s.scan;
     if (w == 0) {
+#endif
         constexpr int EPL = MT / 32;
         uint32_t x[EPL];
         uint32_t sum = 0;
@@ -233,23 +255,35 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
         uint32_t ex = inc - sum;
 #pragma unroll
         for (int q = 0; q < EPL; q++) {
-            s.scan[EPL * L + q] = EPL * L + q < T ? ex : 0xFFFFFFFFu;
-            s.scan[EPL * L + q + MT] = 0xFFFFFFFFu;
+            scan[EPL * L + q] = EPL * L + q < T ? ex : 0xFFFFFFFFu;
+            scan[EPL * L + q + MT] = 0xFFFFFFFFu;
             ex += x[q];
         }
+#if PPR_MS_WSCAN
+        Ew = __shfl_sync(0xffffffffu, inc, 31);
+#else
         if (L == 31) {
             s.E = inc;
             s.chunk = 0;
         }
+#endif
     }
+#if PPR_MS_WSCAN
+    __syncwarp();
+    const uint32_t E = Ew;
+    if (threadIdx.x == 0) s.chunk2[par ^ 1u] = 0;  // the next tile's counter (its last user finished)
+    unsigned int* chunkp = &s.chunk2[par];
+#else
     __syncthreads();
     const uint32_t E = s.E;
+    unsigned int* chunkp = &s.chunk;
+#endif
     // Phase B: warps claim 32-arc chunks of the tile's walk; lane k loads arc k
     // (v, d(v), 1/d(v)) and marks (v, g), then the warp applies the 32 arcs one
     // by one, every lane adding its source's increment to the shared row
     while (true) {
         uint32_t cb = 0;
-        if (L == 0) cb = atomicAdd(&s.chunk, 1u);
+        if (L == 0) cb = atomicAdd(chunkp, 1u);
         cb = __shfl_sync(0xffffffffu, cb, 0);
         if (cb * 32 >= E) break;
         const uint32_t e = cb * 32 + L;
@@ -257,8 +291,8 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
         int j = 0;
         uint32_t v = 0, d = 1;
         if (ok) {
-            j = owner_of(s.scan, e, top);
-            v = ld_pool(&c.pool[s.off[j] + (e - s.scan[j])], pol_stream);
+            j = owner_of(scan, e, top);
+            v = ld_pool(&c.pool[s.off[j] + (e - scan[j])], pol_stream);
             d = ld_dout(&a.g.dout[v], pol_keep);
             mark(a.bitmap, (unsigned long long)v * SG + s.grp[j]);
         }
@@ -274,6 +308,7 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
         }
     }
     __syncthreads();  // smem of this tile is reused by the next
+    c.tiles++;
 }
 
 // every CTA takes tiles of T entries (first statically, the rest by claims)
@@ -288,14 +323,19 @@ __device__ __forceinline__ void ms_round(MsSmem& s, MsCtx& c, const PushArgs& a,
     int top = 1;
     while (top * 2 < (int)T) top <<= 1;
     const uint64_t ntiles = (C + T - 1) / T;
+    const bool dyn = ntiles > gridDim.x;
     uint64_t t = blockIdx.x;
     while (t < ntiles) {
-        ms_tile<POS>(s, c, a, SG, Fin, C, t * T, T, top);
-        if (ntiles <= gridDim.x) break;
-        if (threadIdx.x == 0) s.next = atomicAdd(tc, 1ull) + gridDim.x;
+        // the next tile is claimed as this one starts, so the claim's latency
+        // overlaps the tile (thread 0 first needs the result after it)
+        unsigned long long claim = 0;
+        if (PPR_MS_CLAIM_AHEAD && dyn && threadIdx.x == 0) claim = atomicAdd(tc, 1ull);
+        ms_tile<POS>(s, c, a, SG, Fin, C, t * T, T, top);  // ends with a CTA barrier
+        if (!dyn) break;
+        if (!PPR_MS_CLAIM_AHEAD && threadIdx.x == 0) claim = atomicAdd(tc, 1ull);
+        if (threadIdx.x == 0) s.next = claim + gridDim.x;
         __syncthreads();
-        t = s.next;
-        __syncthreads();
+        t = s.next;  // rewritten only after the next tile's first barrier
     }
 }
 
@@ -396,6 +436,10 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_co
     MsCtx c;
     c.qn = 0;
     c.pushes = c.edges = c.walks = 0;
+    c.tiles = 0;
+#if PPR_MS_WSCAN
+    if (threadIdx.x == 0) s.chunk2[0] = s.chunk2[1] = 0;  // ordered by the grid barrier below
+#endif
     if (*(volatile int*)&a.ctl->st.err != KERR_OK) return;  // earlier stage failed: uniform exit
     c.pool = *(volatile unsigned*)&a.ctl->st.active_pool ? a.g.pool[1] : a.g.pool[0];
     const uint32_t SG = (a.g.S + 31) / 32;

@@ -17,6 +17,11 @@ N > 1  : one process per GPU; rank r maintains its own source (weak scaling:
          S = N sources); rank 0 owns the stream and broadcasts every batch
          over NCCL (the one exchange step), each rank applies it to its graph
          replica.  Step time = max over ranks.
+--sources S : S sources in total (SHARED push with several per rank),
+         partitioned over the ranks by G0 out-degree (dist.partition_sources);
+         value then counts source-edge-updates/s (each update once per source).
+--shard R/G : one process runs only rank R's shard of a G-GPU run of the same
+         sources (the per-rank load of a multi-GPU run, measured on one GPU).
 --impl reference : the CPU oracle (CPU-Seq, 1 thread) on the same workload,
          bounded by --ref-budget-s; rank 0 only.
 """

@@ -487,7 +487,11 @@ ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
         const bool dense = (double)h->m >= 8.0 * (double)h->n;
         a.hyb_all = (a.hyb_thresh && (ha ? atoi(ha) > 0 : dense)) ? 1 : 0;
     }
-    cudaError_t e = launch_push(h->mode, a, h->num_sms, h->st);
+    // dense graphs: 3 edge chains per lane (push_u3.cu); PPR_PUSH_U3=0/1 overrides
+    const char* u3e = getenv("PPR_PUSH_U3");
+    const bool u3 = h->mode == PPR_MODE_OPT && (u3e ? atoi(u3e) > 0 : a.hyb_all != 0);
+    cudaError_t e = u3 ? launch_push_u3(h->mode, a, h->num_sms, h->st)
+                       : launch_push(h->mode, a, h->num_sms, h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, "push launch");
     ++*launches;
     return PPR_OK;

@@ -54,6 +54,9 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_PUSH_U
 #define PPR_PUSH_U 2
 #endif
+#ifndef PPR_PUSH_OPT_ONLY
+#define PPR_PUSH_OPT_ONLY 0
+#endif
 // Opt self-update by exchange: r_u = atomicExch(R(u), 0) (DESIGN.md K-PUSH)
 // per-CTA time split of the trace (PPR_TRACE): compiled in only on request,
 // its counters would otherwise cost registers in every thread
@@ -937,6 +940,9 @@ cudaError_t launch_mode(const PushArgs& a, int num_sms, cudaStream_t st) {
 
 template <bool PK>
 cudaError_t launch_layout(int mode, const PushArgs& a, int num_sms, cudaStream_t st) {
+#if PPR_PUSH_OPT_ONLY
+    return mode == M_OPT ? launch_mode<M_OPT, PK>(a, num_sms, st) : cudaErrorInvalidValue;
+#endif
     switch (mode) {
         case M_OPT: return launch_mode<M_OPT, PK>(a, num_sms, st);
         case M_EAGER: return launch_mode<M_EAGER, PK>(a, num_sms, st);
@@ -950,7 +956,12 @@ cudaError_t launch_layout(int mode, const PushArgs& a, int num_sms, cudaStream_t
 
 }  // namespace
 
-cudaError_t launch_push(int mode, const PushArgs& a, int num_sms, cudaStream_t st) {
+// push_u3.cu compiles this file a second time with 3 edge chains per lane
+// (PPR_PUSH_U=3), Opt only, as launch_push_u3 (dense graphs, ppr_api.cu)
+#ifndef PPR_PUSH_ENTRY
+#define PPR_PUSH_ENTRY launch_push
+#endif
+cudaError_t PPR_PUSH_ENTRY(int mode, const PushArgs& a, int num_sms, cudaStream_t st) {
     if (mode == 6 /* PPR_MODE_SHARED */) return a.g.rec ? cudaErrorInvalidValue : launch_push_ms(a, num_sms, st);
     return a.g.rec ? launch_layout<true>(mode, a, num_sms, st)
                    : launch_layout<false>(mode, a, num_sms, st);

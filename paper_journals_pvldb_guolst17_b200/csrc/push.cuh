@@ -45,6 +45,9 @@ struct PushArgs {
 // Launches the cooperative persistent push kernel for `mode` (PPR_MODE_*).
 cudaError_t launch_push(int mode, const PushArgs& a, int num_sms, cudaStream_t st);
 
+// The Opt push with 3 edge chains per lane (push_u3.cu; dense graphs).
+cudaError_t launch_push_u3(int mode, const PushArgs& a, int num_sms, cudaStream_t st);
+
 // PPR_MODE_SHARED: shared-adjacency multi-source push (push_ms.cu).
 cudaError_t launch_push_ms(const PushArgs& a, int num_sms, cudaStream_t st);
 

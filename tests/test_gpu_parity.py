@@ -146,6 +146,17 @@ def test_opt_schedules_track_oracle(monkeypatch, hyb, hyb_all):
     _run_stream("tiny", "opt", slides=3, sources=3)
 
 
+@pytest.mark.parametrize("hyb,hyb_all", [("0", "0"), ("16384", "1")])
+def test_opt_three_edge_chains_track_oracle(monkeypatch, hyb, hyb_all):
+    # the Opt push compiled with 3 edge chains per lane (push_u3.cu, chosen for
+    # dense graphs) forced on the tiny config, rounds and ring schedules
+    monkeypatch.setenv("PPR_PUSH_U3", "1")
+    monkeypatch.setenv("PPR_HYBRID", hyb)
+    monkeypatch.setenv("PPR_HYBRID_ALL", hyb_all)
+    _run_stream("tiny", "opt", slides=6)
+    _run_stream("tiny", "opt", slides=3, sources=3)
+
+
 @pytest.mark.parametrize("mode", ["opt", "scan", "vanilla"])
 def test_tiny_config_degree_relabelled(mode):
     # internal degree-ordered ids: every id at the boundary must stay external

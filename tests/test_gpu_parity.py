@@ -157,6 +157,16 @@ def test_opt_three_edge_chains_track_oracle(monkeypatch, hyb, hyb_all):
     _run_stream("tiny", "opt", slides=3, sources=3)
 
 
+@pytest.mark.parametrize("mode,hyb_all,relabel", [("opt", "0", -1), ("opt", "1", 1),
+                                                  ("eager", "0", -1), ("vanilla", "0", 1)])
+def test_packed_vertex_records_track_oracle(monkeypatch, mode, hyb_all, relabel):
+    # single-source handles in the packed layout (one 32-byte {R, P, slab, d_out}
+    # record per vertex): same gates as the arrays
+    monkeypatch.setenv("PPR_LAYOUT", "packed")
+    monkeypatch.setenv("PPR_HYBRID_ALL", hyb_all)
+    _run_stream("tiny", mode, slides=8, relabel=relabel)
+
+
 @pytest.mark.parametrize("mode", ["opt", "scan", "vanilla"])
 def test_tiny_config_degree_relabelled(mode):
     # internal degree-ordered ids: every id at the boundary must stay external

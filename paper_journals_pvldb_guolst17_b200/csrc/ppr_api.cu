@@ -680,14 +680,21 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         h->d_dout = reinterpret_cast<uint32_t*>(h->d_hot + Sn);
         h->hot_bytes = sizeof(double) * Sn + sizeof(uint32_t) * h->n;
         // keep R and d_out (the random per-edge targets) resident in L2: the push
-        // is bound by random fp64 atomics, ~3x faster on L2-resident lines
+        // is bound by random fp64 atomics, ~3x faster on L2-resident lines.  Only
+        // when the whole hot set fits the persisting set-aside (LJ 58 MB, Orkut
+        // 37 MB of 79 MB): a window over a larger set (Twitter 480 MB) persists a
+        // random hitRatio share of its lines and slows the push by 18%
+        // (profiles/round1_l2win.md).  PPR_L2_PERSIST=0 / 1 forces it off / on.
         const char* pe = getenv("PPR_L2_PERSIST");
-        if (!(pe && !strcmp(pe, "0"))) {
-            int maxp = 0, maxw = 0;
-            cudaDeviceGetAttribute(&maxp, cudaDevAttrMaxPersistingL2CacheSize, h->device);
-            cudaDeviceGetAttribute(&maxw, cudaDevAttrMaxAccessPolicyWindowSize, h->device);
+        int maxp = 0, maxw = 0;
+        cudaDeviceGetAttribute(&maxp, cudaDevAttrMaxPersistingL2CacheSize, h->device);
+        cudaDeviceGetAttribute(&maxw, cudaDevAttrMaxAccessPolicyWindowSize, h->device);
+        const bool want = pe ? strcmp(pe, "0") != 0 : h->hot_bytes <= (uint64_t)maxp;
+        if (want) {
             if (maxp > 0 && maxw > 0) {
-                const size_t win = std::min<size_t>(h->hot_bytes, (size_t)maxw);
+                size_t win = std::min<size_t>(h->hot_bytes, (size_t)maxw);
+                const char* wm = getenv("PPR_L2_WIN_MB");  // experiment: cap the window (hub prefix of R)
+                if (wm && atof(wm) > 0) win = std::min<size_t>(win, (size_t)(atof(wm) * 1048576.0));
                 const size_t setaside = std::min<size_t>(win, (size_t)maxp);
                 size_t cur = 0;
                 cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize);
@@ -702,6 +709,9 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
                     cudaStreamSetAttribute(h->st, cudaStreamAttributeAccessPolicyWindow, &av) == cudaSuccess;
                 h->l2_win_bytes = win;
                 h->l2_hit = av.accessPolicyWindow.hitRatio;
+                if (getenv("PPR_DEBUG"))
+                    fprintf(stderr, "ppr: L2 window %zu B of %llu hot (max window %d, max set-aside %d), hit ratio %.3f\n",
+                            win, (unsigned long long)h->hot_bytes, maxw, maxp, h->l2_hit);
                 cudaGetLastError();
             }
         }

@@ -196,7 +196,13 @@ __device__ __forceinline__ unsigned lane_id() { return threadIdx.x & 31u; }
 // P, frontiers) with evict_first.
 __device__ __forceinline__ unsigned long long l2_keep() {
     unsigned long long p;
+#if defined(PPR_KEEP_NORMAL)  // experiment builds only
+    asm("createpolicy.fractional.L2::evict_normal.b64 %0, 1.0;" : "=l"(p));
+#elif defined(PPR_KEEP_HALF)
+    asm("createpolicy.fractional.L2::evict_last.L2::evict_unchanged.b64 %0, 0.5;" : "=l"(p));
+#else
     asm("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+#endif
     return p;
 }
 __device__ __forceinline__ unsigned long long l2_stream() {

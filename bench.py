@@ -244,7 +244,7 @@ def config_block(args, cfg, eps, S):
             "undirected": cfg["undirected"], "alpha": 0.15, "eps": eps,
             "source_band": f"top-{cfg['band']} out-degree", "sources": S,
             "rmat_abc": list(cfg["abc"]), "mode": args.mode,
-            "internal_ids": {1: "G0 out-degree order", 0: "external", -1: "auto (degree order iff R+d_out > 48 MB)"}[args.relabel],
+            "internal_ids": {1: "G0 out-degree order", 0: "external", -1: "auto (degree order iff not SHARED and R+d_out > 48 MB)"}[args.relabel],
             "l2": ("persisting lines reset + flushed between steps (512 MiB write)"
                    if not args.no_flush else "not flushed"),
             **({"shard": f"rank {args.shard} of the sources (one GPU's load of a multi-GPU run)"}

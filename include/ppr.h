@@ -110,10 +110,12 @@ typedef struct {
     uint32_t min_cap;    /* minimum slab capacity (default 4) */
     int relabel;         /* 1: vertices are renumbered internally by G0 out-degree (descending)
                             so the most-pushed-to residuals share cache lines; 0: identity;
-                            -1 (default): relabel iff the residual + out-degree arrays
-                            (8*S*n + 4*n bytes) exceed 48 MB, i.e. do not sit in L2 anyway
-                            (measured: LJ-shaped 58 MB -12%, Twitter-shaped -60% per batch;
-                            Orkut-shaped 37 MB +11%, hot lines concentrate on few L2 slices).
+                            -1 (default): relabel iff mode != PPR_MODE_SHARED and the residual
+                            + out-degree arrays (8*S*n + 4*n bytes) exceed 48 MB, i.e. do not sit
+                            in L2 anyway (measured: LJ-shaped 58 MB -12%, Twitter-shaped -60% per
+                            batch, 4 sources in Opt mode -38%; Orkut-shaped 37 MB +11%, hot lines
+                            concentrate on few L2 slices; SHARED 32-source shard +48%, the same
+                            effect on the hubs' S-wide rows).
                             Every id at the boundary stays external. */
 } ppr_opts;
 

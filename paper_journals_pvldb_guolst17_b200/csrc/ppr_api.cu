@@ -756,8 +756,13 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         cudaMemcpyAsync(d_src, g->src, sizeof(uint32_t) * g->m, cudaMemcpyHostToDevice, st);
         cudaMemcpyAsync(d_dst, g->dst, sizeof(uint32_t) * g->m, cudaMemcpyHostToDevice, st);
     }
+    // auto: R + d_out exceed 48 MB, except for the SHARED push: clustering the hubs' S-wide
+    // rows concentrates its row reductions on few L2 slices (32-source shard 37.7 ms relabelled
+    // vs 25.4 ms not; 4 sources in Opt mode 12.3 vs 19.7 ms the other way round;
+    // profiles/round1_spread3.md)
     const bool relabel = o.relabel > 0 ||
-                         (o.relabel < 0 && 8.0 * (double)Sn + 4.0 * h->n > 48.0 * 1024 * 1024);
+                         (o.relabel < 0 && o.mode != PPR_MODE_SHARED &&
+                          8.0 * (double)Sn + 4.0 * h->n > 48.0 * 1024 * 1024);
     if (relabel) {  // degree-ordered internal ids
         uint64_t *k0 = nullptr, *k1 = nullptr;
         uint32_t *v0 = nullptr, *v1 = nullptr, *hist = nullptr;

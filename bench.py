@@ -1,35 +1,42 @@
 #!/usr/bin/env python
 """Benchmark: batch-parallel PPR maintenance on a sliding-window edge stream.
 
-    python bench.py [--gpus N] [--steps K] [--warmup W] [--workload lj]
-                    [--impl ours|reference] [--sources S] [--mode opt]
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--workload lj|ms-lj|orkut|twitter|tiny]
+                    [--impl ours|reference] [--sources S] [--mode auto]
 
-One step = one slide of the window: a batch of 10^4 insertions + 10^4
-deletions (configs[1], LiveJournal-shaped R-MAT) applied through the C ABI
-(ppr_apply_batch): graph-store apply -> invariant restore -> two-phase push
-to eps.  Prints ONE JSON line (rank 0).
+One step = one slide of the window: a batch of insertions + deletions applied
+through the C ABI (ppr_apply_batch): graph-store apply -> invariant restore ->
+two-phase push to eps, for every source the job maintains.  Rank 0 prints ONE
+JSON line.
 
-value  : edge updates/s with the batch already resident in HBM
-         (PPR_MEM_DEVICE), summed over the K timed steps' CUDA-event times.
-e2e    : the same metric through the same call with pinned HOST buffers
-         (H2D of the batch and D2H of the stats inside the timed region).
-N > 1  : one process per GPU; rank r maintains its own source (weak scaling:
-         S = N sources); rank 0 owns the stream and broadcasts every batch
-         over NCCL (the one exchange step), each rank applies it to its graph
-         replica.  Step time = max over ranks.
---sources S : S sources in total (SHARED push with several per rank),
-         partitioned over the ranks by G0 out-degree (dist.partition_sources);
-         value then counts source-edge-updates/s (each update once per source).
---shard R/G : one process runs only rank R's shard of a G-GPU run of the same
-         sources (the per-rank load of a multi-GPU run, measured on one GPU).
---impl reference : the CPU oracle (CPU-Seq, 1 thread) on the same workload,
-         bounded by --ref-budget-s; rank 0 only.
+Workloads (BASELINE.json configs):
+  N = 1 (default)  configs[1]: LiveJournal-shaped, ONE source, 10^4 + 10^4 per
+                   slide.  The line also carries a `multi_source` record:
+                   configs[4] (256 sources) on this one GPU, pushed in waves of
+                   32 sources -- the N = 1 point of the multi-GPU curve.
+  N > 1            configs[4]: the same 256 sources, fixed across N (strong
+                   scaling), dealt to the ranks by G0 out-degree; rank 0 owns
+                   the stream and broadcasts every batch over NCCL (the one
+                   exchange step), every rank applies it to its own graph
+                   replica and maintains its shard.  Launched as one process per
+                   GPU: under torchrun, or -- when WORLD_SIZE is unset -- this
+                   script re-executes itself under torch.distributed.run.
+
+value  : edge updates/s of the whole job (each update counted once, however
+         many sources are maintained) with batches resident in HBM
+         (PPR_MEM_DEVICE).  T = sum over steps of the per-step max over ranks
+         of CUDA-event times on the library's stream; L2 flushed before every
+         step (outside the events).  `source_edge_updates_per_s` = value x S.
+e2e    : the same metric through the same call with pinned HOST buffers (N =
+         1: ppr_apply_batch(PPR_MEM_HOST); N > 1: H2D on rank 0 + the NCCL
+         broadcast) and the D2H of the statistics inside the timed region.
+--impl reference : the CPU oracle (CPU-Seq, 1 thread) on the same workload and
+         slides, bounded by --ref-budget-s; rank 0 only.
 """
 from __future__ import annotations
 
 import argparse
 import json
-import math
 import os
 import statistics
 import subprocess
@@ -42,10 +49,10 @@ import numpy as np
 ROOT = os.path.dirname(os.path.abspath(__file__))
 sys.path.insert(0, ROOT)
 
-# algorithmic bytes per unit: a pushed edge is
-# 24 B = 8 B of walk (v id + d_out(v)) + 16 B of R(v) read+write.  The shared
-# multi-source kernel walks an in-arc once per (source group, arc), so its
-# bytes are 8 per walked arc + 16 per (source, arc) propagation.
+# algorithmic bytes per unit: a pushed edge is 24 B =
+# 8 B of walk (v id + d_out(v)) + 16 B of R(v) read+write; a pushed vertex 52 B.
+# The shared multi-source kernel walks an in-arc once per (source group, arc),
+# so its bytes are 8 per walked arc + 16 per (source, arc) propagation.
 B_EDGE, B_VERTEX, B_ARC = 24, 52, 56
 B_WALK, B_PROP = 8, 16
 
@@ -53,13 +60,16 @@ B_WALK, B_PROP = 8, 16
 def parse():
     p = argparse.ArgumentParser()
     p.add_argument("--gpus", type=int, default=1)
-    p.add_argument("--steps", type=int, default=100)
+    p.add_argument("--steps", type=int, default=20)
     p.add_argument("--warmup", type=int, default=5)
-    p.add_argument("--workload", default="lj")
+    p.add_argument("--workload", default=None,
+                   help="default: lj (configs[1]) at N = 1, ms-lj (configs[4], 256 sources) at N > 1")
     p.add_argument("--impl", default="ours", choices=["ours", "reference"])
-    p.add_argument("--sources", type=int, default=0, help="total sources (0: one per rank)")
+    p.add_argument("--sources", type=int, default=0, help="total sources (0: the workload's)")
     p.add_argument("--mode", default="auto",
-                   help="push mode; auto: opt with one source per rank, scan (EAGER_SCAN) with several")
+                   help="push mode; auto: opt with one source per rank, shared with several")
+    p.add_argument("--wave", type=int, default=32,
+                   help="shared mode: sources per push launch (0: all at once)")
     p.add_argument("--eps", type=float, default=None)
     p.add_argument("--ins", type=int, default=None)
     p.add_argument("--dele", type=int, default=None)
@@ -67,24 +77,30 @@ def parse():
     p.add_argument("--band", type=int, default=None,
                    help="sources drawn from the top-BAND out-degree vertices (default: the config's 1000)")
     p.add_argument("--shard", default=None,
-                   help="R/G: run only rank R's source shard of a G-GPU run on this one GPU "
-                        "(per-rank load of a multi-GPU run; scaling projection)")
+                   help="R/G: run only rank R's source shard of a G-GPU run on this one GPU")
+    p.add_argument("--no-multi-source", action="store_true",
+                   help="N = 1: skip the configs[4] record")
+    p.add_argument("--replica-check-every", type=int, default=10)
     p.add_argument("--no-cpu-baseline", action="store_true")
     p.add_argument("--cpu-budget-s", type=float, default=30.0)
-    p.add_argument("--ref-budget-s", type=float, default=150.0)
+    p.add_argument("--ref-budget-s", type=float, default=120.0)
     p.add_argument("--no-flush", action="store_true")
     p.add_argument("--no-e2e", action="store_true")
     p.add_argument("--backend", default="nccl", choices=["nccl", "gloo"],
-                   help="process-group backend (gloo: test the multi-rank path on one GPU)")
+                   help="process-group backend (gloo: the multi-rank path on one GPU)")
     p.add_argument("--relabel", type=int, default=-1,
                    help="1: degree-ordered internal ids, 0: external ids, -1: by size (default)")
-    return p.parse_args()
+    a = p.parse_args()
+    if a.workload is None:
+        a.workload = "lj" if a.gpus == 1 else "ms-lj"
+    return a
 
 
 # ---------------------------------------------------------------- helpers
 
 class ClockSampler:
-    """nvidia-smi clocks + throttle reasons sampled during the timed region."""
+    """nvidia-smi clocks + throttle reasons, sampled every 50 ms from before the
+    warm-up until after the timed region."""
     Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
          "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
          "clocks_event_reasons.sw_power_cap")
@@ -98,7 +114,7 @@ class ClockSampler:
         try:
             self.proc = subprocess.Popen(
                 ["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.Q}",
-                 "--format=csv,noheader,nounits", "-lms", "200"],
+                 "--format=csv,noheader,nounits", "-lms", "50"],
                 stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
             self.t = threading.Thread(target=self._read, daemon=True)
             self.t.start()
@@ -135,18 +151,18 @@ class ClockSampler:
 def measured_peak():
     try:
         with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
-            return float(json.load(f)["hbm_gbs"]), "measured"
+            return float(json.load(f)["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
     except Exception:
-        return 6650.0, "fallback"
+        return 6650.0, "fallback (B200_PROFILING.md)"
 
 
 def profile_traffic(workload):
-    """dram bytes per push launch from a committed ncu --set full capture, if any."""
+    """DRAM bytes per pushed edge of the push kernel from the committed ncu
+    capture (profiles/push_traffic.json), if any; scaled by the caller."""
     path = os.path.join(ROOT, "profiles", "push_traffic.json")
     try:
         with open(path) as f:
-            d = json.load(f)
-        return d.get(workload, {}).get("dram_bytes_per_launch")
+            return json.load(f).get(workload)
     except Exception:
         return None
 
@@ -164,7 +180,31 @@ def cpu_info():
     return model, os.cpu_count()
 
 
-# ---------------------------------------------------------------- distributed
+def config_block(args, cfg, eps, S, ws):
+    """The workload (identical in both arms' lines)."""
+    return {"workload": args.workload, "n": cfg["n"], "m_stream": cfg["m"],
+            "window": cfg["window"] if cfg["window"] is not None else "resident",
+            "batch": f"{cfg['ins']} ins + {cfg['dele']} del per slide"
+                     + (" (undirected edges)" if cfg["undirected"] else ""),
+            "undirected": cfg["undirected"], "alpha": 0.15, "eps": eps,
+            "source_band": f"top-{cfg['band']} out-degree", "sources": S,
+            "rmat_abc": list(cfg["abc"]), "seed": args.seed,
+            "parallelism": (f"sources dealt over {ws} ranks, graph replicated, batch broadcast"
+                            if ws > 1 else "1 GPU"),
+            "l2": ("persisting lines reset + flushed between steps (512 MiB write)"
+                   if not args.no_flush else "not flushed")}
+
+
+def workload_cfg(args, name):
+    from paper_journals_pvldb_guolst17_b200 import workload as W
+    cfg = dict(W.CONFIGS[name])
+    for k, v in (("ins", args.ins), ("dele", args.dele), ("band", args.band)):
+        if v is not None:
+            cfg[k] = v
+    return cfg
+
+
+# ---------------------------------------------------------------- launch
 
 def dist_env():
     ws = int(os.environ.get("WORLD_SIZE", "1"))
@@ -173,38 +213,59 @@ def dist_env():
     return ws, rank, local
 
 
+def maybe_spawn(args):
+    """--gpus N > 1 without a launcher: re-execute under torch.distributed.run
+    with one process per GPU (rendezvous on 127.0.0.1)."""
+    if "WORLD_SIZE" in os.environ:
+        ws = int(os.environ["WORLD_SIZE"])
+        if ws != args.gpus and not args.shard:
+            raise SystemExit(f"bench.py: WORLD_SIZE={ws} but --gpus {args.gpus}")
+        return
+    if args.gpus <= 1:
+        return
+    import socket
+    with socket.socket() as s:
+        s.bind(("127.0.0.1", 0))
+        port = s.getsockname()[1]
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1",
+           f"--nproc-per-node={args.gpus}", "--master-addr", "127.0.0.1", "--master-port", str(port),
+           os.path.abspath(__file__)] + sys.argv[1:]
+    os.execv(sys.executable, cmd)
+
+
 # ---------------------------------------------------------------- reference arm
 
 def run_reference(args):
+    """The oracle (CPU-Seq, 1 thread) on the same workload and slides: untimed
+    create + static push + W warm-up slides, then timed slides until
+    --ref-budget-s.  With S > 1 sources it maintains one sampled source and
+    reports S x its per-slide time as the job's time (sequential sources)."""
     ws, rank, _ = dist_env()
     if rank != 0:
         return
-    if args.workload == "twitter":
-        print(json.dumps({"impl": "reference", "unavailable": "the sequential oracle cannot build and "
-                          "statically push a 1.5e9-arc window within a bounded sample"}), flush=True)
-        return
     import oracle
     from paper_journals_pvldb_guolst17_b200 import workload as W
-    over = {}
-    if args.ins is not None:
-        over["ins"] = args.ins
-    if args.dele is not None:
-        over["dele"] = args.dele
-    if args.band is not None:
-        over["band"] = args.band
-    st, cfg = W.make_stream(args.workload, seed=args.seed, **over)
+    cfg = workload_cfg(args, args.workload)
     eps = args.eps or cfg["eps"]
+    S = args.sources or cfg["sources"]
+    if args.workload == "twitter":
+        print(json.dumps({"impl": "reference", "unavailable": "the sequential oracle cannot hold and "
+                          "statically push the 1.5e9-arc resident window within a bounded sample"}),
+              flush=True)
+        return
+    over = {k: cfg[k] for k in ("ins", "dele", "band")}
+    st, cfg = W.make_stream(args.workload, seed=args.seed, **over)
     g0s, g0d = st.window()
-    S = args.sources or ws
     srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], S)
     o = oracle.Oracle(cfg["n"], g0s, g0d, srcs[:1], 0.15, eps)
     t0 = time.perf_counter()
     o.push(oracle.SEQ)
     t_static = time.perf_counter() - t0
-    per = []
-    for _ in range(min(args.warmup, 1)):
+    warm = max(args.warmup, 3)
+    for _ in range(warm):
         o.apply(*st.next_batch())
-    for k in range(args.steps):
+    per = []
+    for _ in range(args.steps):
         b = st.next_batch()
         t0 = time.perf_counter()
         o.apply(*b, mode=oracle.SEQ)
@@ -212,298 +273,37 @@ def run_reference(args):
         if sum(per) > args.ref_budget_s:
             break
     upd = cfg["ins"] + cfg["dele"]
-    if cfg["undirected"]:
-        upd = upd  # undirected updates counted as given (not doubled)
-    T = sum(per)
+    T = S * sum(per)  # S sources maintained one after another
     value = upd * len(per) / T
     model, ncpu = cpu_info()
+    sample = (f"{len(per)} timed slides of {cfg['ins']}+{cfg['dele']} after an untimed static push "
+              f"({t_static:.1f} s) and {warm} untimed warm-up slides; "
+              + (f"1 of the {S} sources maintained, job time = {S} x its time; " if S > 1 else "")
+              + f"single thread on {ncpu}-core {model}")
     line = {
         "impl": "reference", "metric": "edge updates/s", "value": value, "unit": "edge updates/s",
-        "n_gpus": args.gpus, "steps": len(per), "warmup": min(args.warmup, 1),
-        "ms_per_step": 1e3 * T / len(per), "higher_is_better": True, "scaling": "weak",
-        "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-        "config": config_block(args, cfg, eps, S),
+        "n_gpus": args.gpus, "steps": len(per), "warmup": warm,
+        "ms_per_step": 1e3 * T / len(per), "higher_is_better": True,
+        "scaling": "strong" if S > 1 else "weak", "vs_baseline": None, "dtype": "f64",
+        "data": "synthetic", "config": config_block(args, cfg, eps, S, max(ws, args.gpus)),
         "cpu_baseline": {"value": value, "unit": "edge updates/s", "cores": 1, "kind": "oracle",
-                         "sample": f"{len(per)} slides of {cfg['ins']}+{cfg['dele']} after an untimed "
-                                   f"static push ({t_static:.1f} s), source rank-band top-{cfg['band']}, "
-                                   f"single thread on {ncpu}-core {model}",
-                         "sources_maintained": 1},
+                         "sample": sample},
         "e2e": {"value": value, "unit": "edge updates/s", "h2d_bytes_per_step": 0,
                 "d2h_bytes_per_step": 0},
     }
-    if S > 1:
-        line["note"] = ("oracle maintains 1 of the S sources; multiply ms_per_step by S for the "
-                        "sequential cost of all sources")
     print(json.dumps(line), flush=True)
-
-
-def config_block(args, cfg, eps, S):
-    return {"workload": args.workload, "n": cfg["n"], "m_stream": cfg["m"],
-            "window": cfg["window"] if cfg["window"] is not None else "resident",
-            "batch": f"{cfg['ins']} ins + {cfg['dele']} del per slide",
-            "undirected": cfg["undirected"], "alpha": 0.15, "eps": eps,
-            "source_band": f"top-{cfg['band']} out-degree", "sources": S,
-            "rmat_abc": list(cfg["abc"]), "mode": args.mode,
-            "internal_ids": {1: "G0 out-degree order", 0: "external", -1: "auto (degree order iff not SHARED and R+d_out > 48 MB)"}[args.relabel],
-            "l2": ("persisting lines reset + flushed between steps (512 MiB write)"
-                   if not args.no_flush else "not flushed"),
-            **({"shard": f"rank {args.shard} of the sources (one GPU's load of a multi-GPU run)"}
-               if getattr(args, "shard", None) else {})}
 
 
 # ---------------------------------------------------------------- our arm
 
-def run_ours(args):
-    import torch
-    import torch.distributed as dist
-
-    from paper_journals_pvldb_guolst17_b200 import dist as D, ppr, workload as W
-
-    ws, rank, local = dist_env()
-    local = local % max(torch.cuda.device_count(), 1)  # several ranks may share a GPU (gloo tests)
-    if ws > 1:
-        if args.backend == "nccl":
-            dist.init_process_group("nccl", device_id=torch.device("cuda", local))
-        else:
-            dist.init_process_group("gloo")
-    torch.cuda.set_device(local)
-    dev = torch.device("cuda", local)
-    stream = torch.cuda.Stream(dev)  # the library runs on this stream; events are recorded on it
-    torch.cuda.set_stream(stream)
-
-    over = {}
-    if args.ins is not None:
-        over["ins"] = args.ins
-    if args.dele is not None:
-        over["dele"] = args.dele
-    if args.band is not None:
-        over["band"] = args.band
-    cfg = dict(W.CONFIGS[args.workload])
-    cfg.update(over)
-    eps = args.eps or cfg["eps"]
-    S = args.sources or ws
-    if S < ws:
-        raise SystemExit("--sources must be >= the world size")
-    steps, warm = args.steps, max(args.warmup, 3)
-    nslides = steps * (1 if args.no_e2e else 2) + warm
-    und = bool(cfg["undirected"])
-    nI, nD = cfg["ins"], cfg["dele"]  # per slide, as given (undirected: edges)
-
-    # rank 0 owns the stream; the window, the sources and every batch reach the
-    # other ranks over NCCL (setup untimed; the per-batch broadcast is timed)
-    t0 = time.perf_counter()
-    if rank == 0:
-        st, cfg = W.make_stream(args.workload, seed=args.seed, **over)
-        g0s, g0d = (st.src[st.lo:st.hi].copy(), st.dst[st.lo:st.hi].copy()) if und else st.window()
-        arcs_s, arcs_d = W.expand_undirected(g0s, g0d) if und else (g0s, g0d)
-        srcs = W.pick_sources(cfg["n"], arcs_s, arcs_d, cfg["band"], S)
-        batches = []
-        for _ in range(nslides):
-            i0, i1 = st.hi, st.hi + nI
-            d0, d1 = st.lo, st.lo + nD
-            if und:  # the library expands undirected edges itself
-                b = (st.src[i0:i1], st.dst[i0:i1], st.src[d0:d1], st.dst[d0:d1])
-                st.hi, st.lo = i1, d1
-            else:
-                b = st.next_batch()
-            batches.append(tuple(np.ascontiguousarray(x) for x in b))
-        meta = torch.tensor([len(g0s)], dtype=torch.int64, device=dev)
-    else:
-        meta = torch.zeros(1, dtype=torch.int64, device=dev)
-    t_gen = time.perf_counter() - t0
-    if ws > 1:
-        dist.broadcast(meta, 0)
-    m0 = int(meta.item())
-    if rank == 0:
-        win = torch.from_numpy(np.stack([g0s, g0d]).view(np.int32)).to(dev)
-        srct = torch.from_numpy(srcs.view(np.int32)).to(dev)
-    else:
-        win = torch.empty((2, m0), dtype=torch.int32, device=dev)
-        srct = torch.empty(S, dtype=torch.int32, device=dev)
-    if ws > 1:
-        dist.broadcast(win, 0)
-        dist.broadcast(srct, 0)
-    win_np = win.cpu().numpy().view(np.uint32)
-    srcs_all = srct.cpu().numpy().view(np.uint32)
-    del win
-    deg = np.bincount(win_np[0], minlength=cfg["n"])
-    if und:
-        deg = deg + np.bincount(win_np[1], minlength=cfg["n"])
-    if args.shard:
-        sr, sg = (int(x) for x in args.shard.split("/"))
-        assert ws == 1 and 0 <= sr < sg, "--shard R/G emulates one rank of G on a single process"
-        my_srcs = D.partition_sources(srcs_all, deg, sg, sr)
-    else:
-        my_srcs = D.partition_sources(srcs_all, deg, ws, rank)
-    if args.mode == "auto":  # measured: Opt best single-source, SHARED for several sources per rank
-        args.mode = "opt" if len(my_srcs) == 1 else "shared"
-
-    t0 = time.perf_counter()
-    h = ppr.Ppr(cfg["n"], win_np[0], win_np[1], my_srcs, alpha=0.15, eps=eps, mode=args.mode,
-                device=local, stream=ctypes_stream(stream), undirected=und,
-                relabel=args.relabel)
-    torch.cuda.synchronize()
-    t_create = time.perf_counter() - t0
-    create_stats = h.create_stats
-    del win_np
-
-    counts = (nI, nD)
-    nflat = 2 * (nI + nD)
-    if rank == 0:
-        dev_batches = [D.pack_batch(*b)[0].to(dev) for b in batches[:warm + steps]]
-    else:
-        dev_batches = [torch.empty(nflat, dtype=torch.int32, device=dev) for _ in range(warm + steps)]
-    flush_buf = torch.empty(512 * 1024 * 1024 // 4, dtype=torch.int32, device=dev)
-
-    def flush():
-        if not args.no_flush:
-            ppr.reset_persisting_l2()  # the handle pins R/d_out in L2; unpin, then evict
-            flush_buf.fill_(1)
-
-    def step_device(flat):
-        flat = D.broadcast_batch(flat, counts)
-        return h.apply_batch(*D.unpack_batch(flat, counts), mem=ppr.MEM_DEVICE)
-
-    for t in range(warm):
-        step_device(dev_batches[t])
-    torch.cuda.synchronize()
-    if ws > 1:
-        dist.barrier()
-
-    # timed: device-resident batches
-    clocks = ClockSampler(local)
-    clocks.start()
-    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
-          for _ in range(steps)]
-    stats = []
-    torch.cuda.synchronize()
-    if ws > 1:
-        dist.barrier()
-    for k in range(steps):
-        flush()
-        ev[k][0].record(stream)
-        stats.append(step_device(dev_batches[warm + k]))
-        ev[k][1].record(stream)
-    torch.cuda.synchronize()
-    if ws > 1:
-        dist.barrier()
-    ms = [a.elapsed_time(b) for a, b in ev]
-
-    # timed: end to end from pinned host buffers through the same call
-    e2e_ms, e2e_stats = [], []
-    if not args.no_e2e:
-        host = []
-        if rank == 0:
-            host = [D.pack_batch(*b)[0].pin_memory() for b in batches[warm + steps:warm + 2 * steps]]
-        buf = torch.empty(nflat, dtype=torch.int32, device=dev)
-        for k in range(steps):
-            flush()
-            a_, b_ = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-            a_.record(stream)
-            if ws > 1:
-                if rank == 0:
-                    buf.copy_(host[k], non_blocking=True)
-                s_ = step_device(buf)
-                s_["h2d_bytes"] = 4 * nflat if rank == 0 else 0
-            else:
-                hb = host[k].numpy().view(np.uint32)
-                s_ = h.apply_batch(*D.unpack_batch(hb, counts), mem=ppr.MEM_HOST)
-            b_.record(stream)
-            b_.synchronize()
-            e2e_ms.append(a_.elapsed_time(b_))
-            e2e_stats.append(s_)
-        torch.cuda.synchronize()
-    clk = clocks.stop()
-
-    # post-run validity: termination (-eps <= R <= eps) for this rank's first source
-    P0, R0 = h.query(0)
-    term_ok = bool(np.all(np.abs(R0) <= eps))
-    term_ok = D.max_over_ranks(0.0 if term_ok else 1.0, device=dev) == 0.0
-
-    T = D.max_over_ranks(sum(ms), device=dev)
-    T_e2e = D.max_over_ranks(sum(e2e_ms), device=dev) if e2e_ms else 0.0
-    push_ms = sum(s["ms_push"] for s in stats)
-    edges_r0 = sum(s["pushed_edges"] for s in stats)
-    verts_r0 = sum(s["pushes"] for s in stats)
-    walks_r0 = sum(s["walk_edges"] for s in stats)
-    edges, verts, launches = D.sum_over_ranks(
-        [edges_r0, verts_r0, sum(s["kernel_launches"] for s in stats)], device=dev)
-    dev_bytes = h.device_bytes
-    h.close()
-    if rank != 0:
-        if ws > 1:
-            dist.destroy_process_group()
-        return
-
-    upd = nI + nD
-    value = S * upd * steps / (T / 1e3)
-    e2e_value = S * upd * len(e2e_ms) / (T_e2e / 1e3) if e2e_ms else None
-    peak, peak_kind = measured_peak()
-    # dominant kernel: the persistent push (one launch per step), rank 0's launches
-    bytes_per_launch = (B_WALK * walks_r0 + B_PROP * edges_r0 + B_VERTEX * verts_r0) / steps
-    push_ms_avg = push_ms / steps
-    achieved = bytes_per_launch / (push_ms_avg / 1e3) / 1e9 if push_ms_avg > 0 else 0.0
-    traffic = profile_traffic(args.workload) if S == 1 else None
-
-    line = {
-        "metric": "edge updates/s", "value": value,
-        "unit": "edge updates/s",  # with S sources each update counts once per source
-        "n_gpus": ws, "steps": steps, "warmup": warm, "ms_per_step": T / steps,
-        "higher_is_better": True, "scaling": "weak" if not args.sources else "strong",
-        "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-        "config": config_block(args, cfg, eps, S),
-        "e2e": ({"value": e2e_value, "unit": "edge updates/s",
-                 "h2d_bytes_per_step": int(np.mean([s["h2d_bytes"] for s in e2e_stats])),
-                 "d2h_bytes_per_step": int(np.mean([s["d2h_bytes"] for s in e2e_stats])),
-                 "ms_per_step": T_e2e / len(e2e_ms)} if e2e_ms else None),
-        "gpu_launches": int(launches),
-        "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                     "frac": achieved / peak, "traffic": traffic,
-                     "kernel": f"k_push<{args.mode.upper()}> (persistent, 1 launch/step)",
-                     "algorithmic_bytes_per_launch": bytes_per_launch,
-                     "peak_kind": peak_kind, "ms_per_launch": push_ms_avg},
-        "clocks": clk,
-        "checks": {"termination_all_ranks": term_ok},
-        "detail": {
-            "ms_per_step_p50": statistics.median(ms), "ms_per_step_p95": float(np.percentile(ms, 95)),
-            "ms_store": sum(s["ms_store"] for s in stats) / steps,
-            "ms_restore": sum(s["ms_restore"] for s in stats) / steps,
-            "ms_push": push_ms_avg,
-            "pushed_edges_per_s": edges / (T / 1e3),
-            "pushes_per_step": verts / steps / S,
-            "pushed_edges_per_step": edges / steps / S,
-            "walk_edges_per_step_rank0": walks_r0 / steps,
-            "iters_per_step": sum(s["iters_pos"] + s["iters_neg"] for s in stats) / steps,
-            "rebuilds": sum(s["rebuilt"] for s in stats),
-            "atomics_per_s_rank0": (edges_r0 + verts_r0) / (push_ms / 1e3) if push_ms else None,
-            "generate_s": t_gen, "create_s": t_create, "create_stats": create_stats,
-            "device_bytes_rank0": dev_bytes, "sources_per_rank": len(my_srcs),
-        },
-    }
-    if not args.no_cpu_baseline and ws == 1 and args.workload == "twitter":
-        line["cpu_baseline"] = {"value": None, "unit": "edge updates/s", "cores": 1, "kind": "oracle",
-                                "unavailable": "the sequential oracle cannot finish the static push of a "
-                                               "1.5e9-arc resident window within a bounded sample"}
-    elif not args.no_cpu_baseline and ws == 1:
-        arcs = (W.expand_undirected(g0s, g0d) if und else (g0s, g0d))
-        bl = [(W.expand_undirected(b[0], b[1]) + W.expand_undirected(b[2], b[3])) if und else b
-              for b in batches]
-        line["cpu_baseline"] = cpu_baseline(args, cfg, eps, my_srcs[:1], arcs[0], arcs[1], bl)
-    print(json.dumps(line), flush=True)
-    if ws > 1:
-        dist.destroy_process_group()
-
-
-def ctypes_stream(stream):
-    return stream.cuda_stream
-
-
-def cpu_baseline(args, cfg, eps, srcs, g0s, g0d, batches):
-    """The oracle (as it stands, CPU-Seq, 1 thread) on a bounded sample of the
-    same workload: untimed create + static push on the same window, then the
-    same slides, timed until --cpu-budget-s is used."""
+def cpu_baseline(args, cfg, eps, srcs, g0s, g0d, batches, warm, S_job):
+    """The oracle as it stands (CPU-Seq, 1 thread) on a bounded sample of the
+    same workload: untimed create + static push, then the stream's first
+    slides, timed until --cpu-budget-s (no warm-up slides: each costs seconds
+    on one core).  S_job > 1: it maintains srcs[:1] and the job's time is
+    S_job x its time."""
     import oracle
-    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, eps)
+    o = oracle.Oracle(cfg["n"], g0s, g0d, srcs[:1], 0.15, eps)
     t0 = time.perf_counter()
     o.push(oracle.SEQ)
     t_static = time.perf_counter() - t0
@@ -516,16 +316,360 @@ def cpu_baseline(args, cfg, eps, srcs, g0s, g0d, batches):
             break
     model, ncpu = cpu_info()
     upd = cfg["ins"] + cfg["dele"]
-    return {"value": upd * len(per) / sum(per), "unit": "edge updates/s", "cores": 1,
-            "kind": "oracle",
-            "sample": f"first {len(per)} slides of the same stream and source (rank 0's), "
-                      f"after an untimed static push of {t_static:.1f} s; 1 thread of "
-                      f"{ncpu}-core {model}",
-            "ms_per_step": 1e3 * sum(per) / len(per)}
+    T = S_job * sum(per)
+    return {"value": upd * len(per) / T, "unit": "edge updates/s", "cores": 1, "kind": "oracle",
+            "sample": f"the first {len(per)} timed slides of the same stream"
+                      + (f", 1 sampled source of {S_job} (job time = {S_job} x its time)" if S_job > 1
+                         else ", same source")
+                      + f", after an untimed static push of {t_static:.1f} s; 1 thread of "
+                        f"{ncpu}-core {model}",
+            "ms_per_step": 1e3 * T / len(per)}
+
+
+class Ctx:
+    """Process-group / device context of this rank."""
+
+    def __init__(self, args):
+        import torch
+        import torch.distributed as dist
+        self.ws, self.rank, local = dist_env()
+        self.local = local % max(torch.cuda.device_count(), 1)  # ranks may share a GPU (gloo)
+        self.dist_on = self.ws > 1
+        if self.dist_on:
+            if args.backend == "nccl":
+                dist.init_process_group("nccl", device_id=torch.device("cuda", self.local))
+            else:
+                dist.init_process_group("gloo")
+            assert dist.get_world_size() == self.ws
+        torch.cuda.set_device(self.local)
+        self.dev = torch.device("cuda", self.local)
+        self.stream = torch.cuda.Stream(self.dev)  # the library runs (and is timed) on this stream
+        torch.cuda.set_stream(self.stream)
+        self.comm_dev = self.dev if args.backend == "nccl" else torch.device("cpu")
+
+    def bcast(self, t):
+        import torch.distributed as dist
+        if not self.dist_on:
+            return t
+        if self.comm_dev.type == "cpu" and t.is_cuda:
+            c = t.cpu()
+            dist.broadcast(c, 0)
+            t.copy_(c)
+        else:
+            dist.broadcast(t, 0)
+        return t
+
+    def barrier(self):
+        import torch.distributed as dist
+        if self.dist_on:
+            dist.barrier()
+
+    def max_vec(self, xs):
+        import torch
+        import torch.distributed as dist
+        t = torch.tensor(list(xs), dtype=torch.float64, device=self.comm_dev)
+        if self.dist_on:
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        return t.tolist()
+
+    def sum_vec(self, xs):
+        import torch
+        import torch.distributed as dist
+        t = torch.tensor([float(x) for x in xs], dtype=torch.float64, device=self.comm_dev)
+        if self.dist_on:
+            dist.all_reduce(t, op=dist.ReduceOp.SUM)
+        return t.tolist()
+
+
+def measure(args, cx, workload, S_total, with_e2e, with_cpu):
+    """Runs one workload on this rank and returns the rank-0 record (None on
+    other ranks): create, W warm-up slides, K timed device-resident slides,
+    K timed e2e slides."""
+    import torch
+
+    from paper_journals_pvldb_guolst17_b200 import dist as D, ppr, workload as W
+
+    cfg = workload_cfg(args, workload)
+    eps = args.eps or cfg["eps"]
+    und = bool(cfg["undirected"])
+    nI, nD = cfg["ins"], cfg["dele"]
+    steps, warm = args.steps, max(args.warmup, 3)
+    nslides = warm + steps * (2 if with_e2e else 1)
+    dev = cx.dev
+
+    # rank 0 owns the stream; window, sources and batches reach the other ranks
+    # over the process group (setup untimed; the per-batch broadcast is timed)
+    t0 = time.perf_counter()
+    batches = []
+    if cx.rank == 0:
+        over = {k: cfg[k] for k in ("ins", "dele", "band")}
+        st, cfg = W.make_stream(workload, seed=args.seed, **over)
+        g0s, g0d = (st.src[st.lo:st.hi].copy(), st.dst[st.lo:st.hi].copy()) if und else st.window()
+        arcs_s, arcs_d = W.expand_undirected(g0s, g0d) if und else (g0s, g0d)
+        srcs = W.pick_sources(cfg["n"], arcs_s, arcs_d, cfg["band"], S_total)
+        for _ in range(nslides):
+            i0, i1, d0, d1 = st.hi, st.hi + nI, st.lo, st.lo + nD
+            if und:  # the library expands undirected edges itself
+                b = (st.src[i0:i1], st.dst[i0:i1], st.src[d0:d1], st.dst[d0:d1])
+                st.hi, st.lo = i1, d1
+            else:
+                b = st.next_batch()
+            batches.append(tuple(np.ascontiguousarray(x) for x in b))
+        meta = torch.tensor([len(g0s)], dtype=torch.int64, device=dev)
+    else:
+        meta = torch.zeros(1, dtype=torch.int64, device=dev)
+    t_gen = time.perf_counter() - t0
+    cx.bcast(meta)
+    m0 = int(meta.item())
+    if cx.rank == 0:
+        win = torch.from_numpy(np.stack([g0s, g0d]).view(np.int32)).to(dev)
+        srct = torch.from_numpy(srcs.view(np.int32)).to(dev)
+    else:
+        win = torch.empty((2, m0), dtype=torch.int32, device=dev)
+        srct = torch.empty(S_total, dtype=torch.int32, device=dev)
+    cx.bcast(win)
+    cx.bcast(srct)
+    win_np = win.cpu().numpy().view(np.uint32)
+    srcs_all = srct.cpu().numpy().view(np.uint32)
+    del win
+    deg = np.bincount(win_np[0], minlength=cfg["n"])
+    if und:
+        deg = deg + np.bincount(win_np[1], minlength=cfg["n"])
+    if args.shard:
+        sr, sg = (int(x) for x in args.shard.split("/"))
+        assert cx.ws == 1 and 0 <= sr < sg, "--shard R/G emulates one rank of G on a single process"
+        my_srcs = D.partition_sources(srcs_all, deg, sg, sr)
+    else:
+        my_srcs = D.partition_sources(srcs_all, deg, cx.ws, cx.rank)
+    mode = args.mode
+    if mode == "auto":  # measured: Opt best for one source per rank, SHARED for several
+        mode = "opt" if len(my_srcs) == 1 else "shared"
+    wave = args.wave if (mode == "shared" and args.wave and len(my_srcs) > args.wave) else 0
+
+    t0 = time.perf_counter()
+    h = ppr.Ppr(cfg["n"], win_np[0], win_np[1], my_srcs, alpha=0.15, eps=eps, mode=mode,
+                device=cx.local, stream=cx.stream.cuda_stream, undirected=und,
+                relabel=args.relabel)
+    if wave:
+        h.set_option(ppr.OPT_WAVE, wave)
+    torch.cuda.synchronize()
+    t_create = time.perf_counter() - t0
+    create_stats = h.create_stats
+    del win_np
+
+    counts = (nI, nD)
+    nflat = 2 * (nI + nD)
+    if cx.rank == 0:
+        dev_batches = [D.pack_batch(*b)[0].to(dev) for b in batches[:warm + steps]]
+    else:
+        dev_batches = [torch.empty(nflat, dtype=torch.int32, device=dev) for _ in range(warm + steps)]
+    flush_buf = torch.empty(512 * 1024 * 1024 // 4, dtype=torch.int32, device=dev)
+
+    def flush():
+        if not args.no_flush:
+            ppr.reset_persisting_l2()  # persisting lines back to normal, then evicted
+            flush_buf.fill_(1)
+
+    def step_device(flat):
+        cx.bcast(flat)
+        return h.apply_batch(*D.unpack_batch(flat, counts), mem=ppr.MEM_DEVICE)
+
+    replica_checks = []
+
+    def replica_check():
+        gs, gd = h.export_edges()
+        ok = D.replicas_agree(D.edge_set_digest(gs, gd), device=cx.comm_dev)
+        replica_checks.append(bool(ok))
+
+    clocks = ClockSampler(cx.local)
+    clocks.start()
+    for t in range(warm):
+        step_device(dev_batches[t])
+    torch.cuda.synchronize()
+    cx.barrier()
+
+    # timed: device-resident batches, each step bracketed by CUDA events on the
+    # library's stream; flush and replica checks between steps, outside them
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
+          for _ in range(steps)]
+    stats = []
+    for k in range(steps):
+        flush()
+        ev[k][0].record(cx.stream)
+        stats.append(step_device(dev_batches[warm + k]))
+        ev[k][1].record(cx.stream)
+        if cx.dist_on and args.replica_check_every and (k + 1) % args.replica_check_every == 0:
+            torch.cuda.synchronize()
+            replica_check()
+    torch.cuda.synchronize()
+    cx.barrier()
+    ms = [a.elapsed_time(b) for a, b in ev]
+
+    # timed: end to end from pinned host buffers through the same call
+    e2e_ms, e2e_stats = [], []
+    if with_e2e:
+        host = []
+        if cx.rank == 0:
+            host = [D.pack_batch(*b)[0].pin_memory() for b in batches[warm + steps:warm + 2 * steps]]
+        buf = torch.empty(nflat, dtype=torch.int32, device=dev)
+        for k in range(steps):
+            flush()
+            a_, b_ = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a_.record(cx.stream)
+            if cx.dist_on:
+                if cx.rank == 0:
+                    buf.copy_(host[k], non_blocking=True)
+                s_ = step_device(buf)
+                s_["h2d_bytes"] = 4 * nflat if cx.rank == 0 else 0
+            else:
+                hb = host[k].numpy().view(np.uint32)
+                s_ = h.apply_batch(*D.unpack_batch(hb, counts), mem=ppr.MEM_HOST)
+            b_.record(cx.stream)
+            b_.synchronize()
+            e2e_ms.append(a_.elapsed_time(b_))
+            e2e_stats.append(s_)
+        torch.cuda.synchronize()
+    clk = clocks.stop()
+
+    # post-run validity: termination (-eps <= R <= eps) for every source of this rank
+    term_ok = all(bool(np.all(np.abs(h.query(i)[1]) <= eps)) for i in range(len(my_srcs)))
+    if cx.dist_on:
+        replica_check()
+    dev_bytes = h.device_bytes
+    h.close()
+
+    # per-step max over ranks, summed: T = sum_k max_r t_{k,r}
+    ms_max = cx.max_vec(ms)
+    T = sum(ms_max)
+    e2e_max = cx.max_vec(e2e_ms) if e2e_ms else []
+    T_e2e = sum(e2e_max)
+    push_ms = [s["ms_push"] for s in stats]
+    keys = ["pushed_edges", "pushes", "walk_edges", "kernel_launches"]
+    tot = dict(zip(keys, cx.sum_vec([sum(s[k] for s in stats) for k in keys])))
+    ok_all = cx.sum_vec([0.0 if term_ok else 1.0, float(sum(not x for x in replica_checks))])
+    if cx.rank != 0:
+        return None
+
+    upd = nI + nD
+    value = upd * steps / (T / 1e3)
+    peak, peak_kind = measured_peak()
+    # dominant kernel: the persistent push (one launch per step, or one per
+    # source wave), rank 0's launches, timed by the library's events on its stream
+    n_launch = 1 if not wave else -(-len(my_srcs) // wave)
+    e_r0 = sum(s["pushed_edges"] for s in stats) / steps
+    v_r0 = sum(s["pushes"] for s in stats) / steps
+    w_r0 = sum(s["walk_edges"] for s in stats) / steps
+    bytes_step = (B_WALK * w_r0 + B_PROP * e_r0 + B_VERTEX * v_r0)
+    push_step = sum(push_ms) / steps
+    achieved = bytes_step / (push_step / 1e3) / 1e9 if push_step > 0 else 0.0
+    tr = profile_traffic(workload) if len(my_srcs) == 1 else None
+    traffic = None
+    if tr and tr.get("dram_bytes_per_pushed_edge"):
+        traffic = tr["dram_bytes_per_pushed_edge"] * e_r0 / n_launch
+    rec = {
+        "value": value, "ms_per_step": T / steps,
+        "source_edge_updates_per_s": value * S_total,
+        "config": config_block(args, cfg, eps, S_total, cx.ws),
+        "impl_config": {"mode": mode, "sources_per_rank": len(my_srcs), "wave": wave or None,
+                        "internal_ids": {1: "G0 out-degree order", 0: "external",
+                                         -1: "auto (degree order iff not SHARED and R+d_out > 48 MB)"
+                                         }[args.relabel]},
+        "e2e": ({"value": upd * len(e2e_ms) / (T_e2e / 1e3), "unit": "edge updates/s",
+                 "h2d_bytes_per_step": int(np.mean([s["h2d_bytes"] for s in e2e_stats])),
+                 "d2h_bytes_per_step": int(np.mean([s["d2h_bytes"] for s in e2e_stats])),
+                 "ms_per_step": T_e2e / len(e2e_ms)} if e2e_ms else None),
+        "gpu_launches": int(tot["kernel_launches"]),
+        "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                     "frac": achieved / peak, "traffic": traffic,
+                     "kernel": f"k_push<{mode.upper()}> (persistent, {n_launch} launch(es)/step)",
+                     "algorithmic_bytes_per_launch": bytes_step / n_launch,
+                     "ms_per_launch": push_step / n_launch, "peak_kind": peak_kind,
+                     "traffic_source": (tr or {}).get("source")},
+        "clocks": clk,
+        "checks": {"termination_all_ranks_all_sources": ok_all[0] == 0.0,
+                   "replica_checks": len(replica_checks), "replicas_agree": ok_all[1] == 0.0},
+        "detail": {
+            "ms_per_step_p50": statistics.median(ms_max),
+            "ms_per_step_p95": float(np.percentile(ms_max, 95)),
+            "ms_store": sum(s["ms_store"] for s in stats) / steps,
+            "ms_restore": sum(s["ms_restore"] for s in stats) / steps,
+            "ms_push": push_step,
+            "ms_push_pos": sum(s["ms_push_pos"] for s in stats) / steps,
+            "ms_push_neg": sum(s["ms_push_neg"] for s in stats) / steps,
+            "pushed_edges_per_s": tot["pushed_edges"] / (T / 1e3),
+            "pushes_per_step": tot["pushes"] / steps,
+            "pushed_edges_per_step": tot["pushed_edges"] / steps,
+            "iters_per_step": sum(s["iters_pos"] + s["iters_neg"] for s in stats) / steps,
+            "rebuilds": sum(s["rebuilt"] for s in stats),
+            "generate_s": t_gen, "create_s": t_create, "create_stats": create_stats,
+            "device_bytes_rank0": dev_bytes,
+            # rank 0's own timed slides, in order (slide index = warm-up + k): the ncu
+            # capture of the same launch is matched against these (profiles/)
+            "per_step_rank0": [{"slide": warm + k, "ms": round(ms[k], 4),
+                                "ms_push": round(s["ms_push"], 4), "pushed_edges": s["pushed_edges"],
+                                "pushes": s["pushes"], "iters": s["iters_pos"] + s["iters_neg"]}
+                               for k, s in enumerate(stats)],
+        },
+    }
+    if with_cpu and not args.no_cpu_baseline:
+        if workload == "twitter":
+            rec["cpu_baseline"] = {"value": None, "unit": "edge updates/s", "cores": 1, "kind": "oracle",
+                                   "unavailable": "the sequential oracle cannot hold and statically push "
+                                                  "the 1.5e9-arc resident window within a bounded sample"}
+        else:
+            arcs = (W.expand_undirected(g0s, g0d) if und else (g0s, g0d))
+            bl = [(W.expand_undirected(b[0], b[1]) + W.expand_undirected(b[2], b[3])) if und else b
+                  for b in batches]
+            rec["cpu_baseline"] = cpu_baseline(args, cfg, eps, srcs, arcs[0], arcs[1], bl, warm,
+                                               S_total)
+    return rec
+
+
+def run_ours(args):
+    import torch.distributed as dist
+    cx = Ctx(args)
+    cfg = workload_cfg(args, args.workload)
+    S = args.sources or cfg["sources"]
+    if S < cx.ws:
+        raise SystemExit("--sources must be >= the world size")
+    rec = measure(args, cx, args.workload, S, with_e2e=not args.no_e2e, with_cpu=cx.ws == 1)
+    multi = None
+    if cx.ws == 1 and args.workload == "lj" and not args.no_multi_source and not args.shard:
+        # the N = 1 point of the configs[4] curve (256 sources on this GPU, in waves)
+        wl = args.workload
+        args.workload = "ms-lj"
+        multi = measure(args, cx, "ms-lj", workload_cfg(args, "ms-lj")["sources"], with_e2e=False,
+                        with_cpu=True)
+        args.workload = wl
+    if cx.rank == 0:
+        line = {"metric": "edge updates/s", "value": rec["value"], "unit": "edge updates/s",
+                "n_gpus": cx.ws, "steps": args.steps, "warmup": max(args.warmup, 3),
+                "ms_per_step": rec["ms_per_step"], "higher_is_better": True,
+                "scaling": "strong" if S > 1 else "weak", "vs_baseline": None, "dtype": "f64",
+                "data": "synthetic"}
+        line.update({k: v for k, v in rec.items() if k not in ("value", "ms_per_step")})
+        if multi is not None:
+            line["multi_source"] = {
+                "what": "configs[4]: 256 sources on this one GPU (the N = 1 point of the strong-scaling "
+                        "curve that bench.py --gpus N measures as its headline)",
+                "metric": "edge updates/s", "value": multi["value"], "unit": "edge updates/s",
+                "ms_per_step": multi["ms_per_step"],
+                "source_edge_updates_per_s": multi["source_edge_updates_per_s"],
+                "config": multi["config"], "impl_config": multi["impl_config"],
+                "roofline": multi["roofline"], "checks": multi["checks"],
+                "cpu_baseline": multi.get("cpu_baseline"),
+                "detail": {k: multi["detail"][k] for k in
+                           ("ms_store", "ms_restore", "ms_push", "ms_push_pos", "ms_push_neg",
+                            "pushed_edges_per_step", "pushes_per_step", "iters_per_step")},
+            }
+        print(json.dumps(line), flush=True)
+    if cx.dist_on:
+        dist.destroy_process_group()
 
 
 def main():
     args = parse()
+    maybe_spawn(args)
     if args.impl == "reference":
         run_reference(args)
     else:

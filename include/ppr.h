@@ -117,7 +117,16 @@ typedef struct {
                             concentrate on few L2 slices; SHARED 32-source shard +48%, the same
                             effect on the hubs' S-wide rows).
                             Every id at the boundary stays external. */
+    int layout;          /* PPR_LAYOUT_ARRAYS (default): R / d_out / slab / P as separate arrays;
+                            PPR_LAYOUT_PACKED: one 32-byte {R, P, off, len, d_out, cap} record per
+                            vertex (single source, not SHARED / SORTAGG, pool < 2^32 entries;
+                            otherwise PPR_EINVAL).  Measured slower on every shape. */
+    int l2_persist;      /* persisting L2 access-policy window over R and d_out, passed with each
+                            push launch: -1 (default) iff they fit the device's persisting
+                            set-aside, 0 never, 1 always */
 } ppr_opts;
+
+enum { PPR_LAYOUT_ARRAYS = 0, PPR_LAYOUT_PACKED = 1 };
 
 /* Per-call statistics (filled by ppr_create, ppr_apply_batch, ppr_push). */
 typedef struct {
@@ -131,10 +140,17 @@ typedef struct {
     uint32_t kernel_launches;       /* kernels launched by this call */
     uint64_t h2d_bytes, d2h_bytes;  /* host<->device bytes this call copied */
     float ms_total;                 /* CUDA-event time of the call on the stream */
-    float ms_store, ms_restore, ms_push; /* per phase (0 if timing disabled) */
+    float ms_store;                 /* CUDA events: batch staging through the store and restore
+                                       branches (a0-a2; the restore branch runs concurrently) */
+    float ms_restore;               /* device clock (%globaltimer): the Lemma 3 restore kernel
+                                       alone (a2), first CTA start to last CTA end; inside ms_store */
+    float ms_push;                  /* CUDA events around the push launch (a3-a6, both phases) */
     uint64_t walk_edges;            /* in-arc reads of the push: PPR_MODE_SHARED walks N_in(u) once
                                        per (source group, u), so walk_edges <= pushed_edges;
                                        other modes: = pushed_edges */
+    float ms_push_pos, ms_push_neg; /* device clock inside the push launch: seed + rounds of the
+                                       POS phase (a3-a4) and of the NEG phase (a5); 0 for
+                                       PPR_MODE_SORTAGG (host-driven rounds) */
 } ppr_batch_stats;
 
 /* Creates a handle: builds the slab store for g, sets P_s = 0 and R_s = e_s
@@ -182,7 +198,21 @@ enum {
     PPR_OPT_PUSH = 2,      /* 0: ppr_apply_batch stops after restore (tests); default 1 */
     PPR_OPT_MAX_ITERS = 3, /* stop each phase after this many rounds (0 = run to eps) */
     PPR_OPT_TIMING = 4,    /* 1: record per-phase CUDA events (default 1) */
-    PPR_OPT_FORCE_REBUILD = 5 /* 1: every batch takes the sort/merge rebuild path */
+    PPR_OPT_FORCE_REBUILD = 5, /* 1: every batch takes the sort/merge rebuild path */
+    PPR_OPT_RING_TAIL = 6,   /* Opt: a phase whose frontier has shrunk (past its peak) to at most
+                                this many entries finishes on the asynchronous ring worklist
+                                (default 16384; 0: rounds to the end) */
+    PPR_OPT_RING_ALL = 7,    /* Opt: whole phases on the ring from their seeds: -1 (default) iff
+                                the graph has >= 8 arcs per vertex, 0 never, 1 always
+                                (needs RING_TAIL > 0) */
+    PPR_OPT_EDGE_CHAINS = 8, /* Opt: independent edge chains per lane, 2 or 3 (0 = default: 3
+                                when whole phases run on the ring, else 2) */
+    PPR_OPT_GRAPHS = 9,      /* 1 (default): replay each batch shape's store/restore pipeline as
+                                one CUDA graph; 0: launch the kernels one by one */
+    PPR_OPT_WAVE = 10        /* PPR_MODE_SHARED: push the sources in waves of this many (a
+                                multiple of 32; 0 = default: all in one launch), one push launch
+                                per wave after the shared store/restore, so each launch's residual
+                                rows stay L2-sized */
 };
 ppr_status ppr_set_option(ppr_ctx *h, int key, int64_t value);
 

@@ -22,6 +22,8 @@
 #include <cstdio>
 #include <cstdlib>
 #include <cstring>
+#include <map>
+#include <mutex>
 #include <new>
 #include <string>
 #include <vector>
@@ -44,11 +46,12 @@ struct GraphKey {
     uint64_t epoch = 0, cap0 = 0, cap1 = 0;
     const void* pool0 = nullptr;
     const void* pool1 = nullptr;
+    unsigned active = 0;  // the rebuild's capacity check (StoreParams::alt_cap) is baked in per active pool
     bool operator==(const GraphKey& o) const {
         return n_ins == o.n_ins && n_del == o.n_del && push == o.push && mode == o.mode &&
                max_iters == o.max_iters && timing == o.timing && force_rebuild == o.force_rebuild &&
                epoch == o.epoch && cap0 == o.cap0 && cap1 == o.cap1 && pool0 == o.pool0 &&
-               pool1 == o.pool1;
+               pool1 == o.pool1 && active == o.active;
     }
 };
 
@@ -113,12 +116,64 @@ struct ppr_ctx {
     unsigned long long* d_ring = nullptr;   // PPR_MODE_ASYNC ring queue (2*S*n slots, EMPTY)
     unsigned long long ring_cap = 0;
     uint64_t hyb_thresh = 0;                // Opt: frontier size at which a phase finishes on the ring
+    int ring_all = -1;                      // Opt: whole phases on the ring (-1: iff >= 8 arcs per vertex)
+    int edge_chains = 0;                    // Opt: edge chains per lane (0: 3 iff ring_all, else 2)
+    uint32_t wave = 0;                      // SHARED: sources per push launch (multiple of 32; 0: all)
     unsigned long long* d_trace = nullptr;  // PPR_TRACE=1: per-round trace of the push
     uint32_t trace_cap = 0;
     SortAgg* sa = nullptr;                  // PPR_MODE_SORTAGG scratch (grown on demand)
 };
 
 namespace {
+
+bool dbg_on() {  // PPR_DEBUG=1: report launch errors / L2 setup on stderr (diagnostics only)
+    static const bool on = getenv("PPR_DEBUG") && atoi(getenv("PPR_DEBUG")) > 0;
+    return on;
+}
+
+// Persisting-L2 set-aside per device, reference-counted over the handles that
+// use an access-policy window: the first raises cudaLimitPersistingL2CacheSize
+// (remembering the previous value), the last restores it.  Persisting lines
+// of other handles are never reset here.
+struct L2Share {
+    int refs = 0;
+    size_t prev = 0, cur = 0;
+};
+std::mutex g_l2_mu;
+std::map<int, L2Share> g_l2;
+
+bool l2_acquire(int device, size_t bytes) {
+    std::lock_guard<std::mutex> lk(g_l2_mu);
+    L2Share& s = g_l2[device];
+    size_t cur = 0;
+    if (cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize) != cudaSuccess) {
+        cudaGetLastError();
+        return false;
+    }
+    if (s.refs == 0) s.prev = cur;
+    if (cur < bytes && cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, bytes) != cudaSuccess) {
+        cudaGetLastError();
+        return false;
+    }
+    s.cur = std::max(cur, bytes);
+    s.refs++;
+    return true;
+}
+
+void l2_release(int device) {
+    std::lock_guard<std::mutex> lk(g_l2_mu);
+    auto it = g_l2.find(device);
+    if (it == g_l2.end() || it->second.refs == 0) return;
+    if (--it->second.refs == 0) {
+        int cur_dev = 0;
+        cudaGetDevice(&cur_dev);
+        cudaSetDevice(device);
+        cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, it->second.prev);
+        cudaSetDevice(cur_dev);
+        cudaGetLastError();
+        g_l2.erase(it);
+    }
+}
 
 void set_err(ppr_ctx* h, const char* fmt, ...) {
     char buf[512];
@@ -282,11 +337,13 @@ void fill_stats(ppr_ctx* h, ppr_batch_stats* s, uint32_t launches, bool timed,
         s->ms_total = ms;
         cudaEventElapsedTime(&ms, h->ev[0], h->ev[1]);
         s->ms_store = ms;
-        cudaEventElapsedTime(&ms, h->ev[1], h->ev[2]);
-        s->ms_restore = ms;
         cudaEventElapsedTime(&ms, h->ev[2], h->ev[3]);
         s->ms_push = ms;
     }
+    // device-clock phase times (DevStats stamps; 0 where the stage did not run)
+    if (c.t_restore[1] > c.t_restore[0]) s->ms_restore = (float)((c.t_restore[1] - c.t_restore[0]) * 1e-6);
+    s->ms_push_pos = (float)(c.ns_push[0] * 1e-6);
+    s->ms_push_neg = (float)(c.ns_push[1] * 1e-6);
 }
 
 PushArgs push_args(ppr_ctx* h) {
@@ -361,7 +418,7 @@ ppr_status finish(ppr_ctx* h, const char* where) {
 void record(ppr_ctx* h, int i) {
     if (h->timing) {
         cudaError_t e = cudaEventRecord(h->ev[i], h->st);
-        if (e != cudaSuccess && getenv("PPR_DEBUG"))
+        if (e != cudaSuccess && dbg_on())
             fprintf(stderr, "PPR_DEBUG: event record %d: %s\n", i, cudaGetErrorString(e));
     }
 }
@@ -371,11 +428,8 @@ void destroy_all(ppr_ctx* h) {
     if (h->gexec) cudaGraphExecDestroy(h->gexec), h->gexec = nullptr;
     free_batch(h);
     dfree(h, h->d_rec, h->n);
-    if (h->l2_window && h->st) {  // drop the window from the (possibly caller's) stream
-        cudaStreamAttrValue av{};
-        av.accessPolicyWindow.num_bytes = 0;
-        cudaStreamSetAttribute(h->st, cudaStreamAttributeAccessPolicyWindow, &av);
-        cudaCtxResetPersistingL2Cache();
+    if (h->l2_window) {
+        l2_release(h->device);
         h->l2_window = false;
     }
     if (h->d_hot) {
@@ -420,6 +474,9 @@ void destroy_all(ppr_ctx* h) {
     if (h->own_stream && h->st) cudaStreamDestroy(h->st);
     h->st = nullptr;
 }
+
+constexpr uint64_t kRingTailDefault = 16384;  // entries
+bool ring_fits(const ppr_ctx* h) { return (uint64_t)h->S * h->n <= (1ull << 27); }
 
 ppr_status ensure_ring(ppr_ctx* h) {
     if (h->d_ring) return PPR_OK;
@@ -483,17 +540,23 @@ ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
     // dense graphs (>= 8 arcs per vertex) push on the ring from the start: rounds
     // there only add barriers, no accumulation
     {
-        const char* ha = getenv("PPR_HYBRID_ALL");
         const bool dense = (double)h->m >= 8.0 * (double)h->n;
-        a.hyb_all = (a.hyb_thresh && (ha ? atoi(ha) > 0 : dense)) ? 1 : 0;
+        a.hyb_all = (a.hyb_thresh && (h->ring_all < 0 ? dense : h->ring_all > 0)) ? 1 : 0;
     }
-    // dense graphs: 3 edge chains per lane (push_u3.cu); PPR_PUSH_U3=0/1 overrides
-    const char* u3e = getenv("PPR_PUSH_U3");
-    const bool u3 = h->mode == PPR_MODE_OPT && (u3e ? atoi(u3e) > 0 : a.hyb_all != 0);
-    cudaError_t e = u3 ? launch_push_u3(h->mode, a, h->num_sms, h->st)
-                       : launch_push(h->mode, a, h->num_sms, h->st);
-    if (e != cudaSuccess) return cuda_fail(h, e, "push launch");
-    ++*launches;
+    // dense graphs: 3 edge chains per lane (push_u3.cu); PPR_OPT_EDGE_CHAINS overrides
+    const bool u3 = h->mode == PPR_MODE_OPT && (h->edge_chains == 0 ? a.hyb_all != 0 : h->edge_chains == 3);
+    // SHARED with a wave size: one launch per group of wave/32 source groups, so
+    // each launch's residual rows stay L2-sized (PPR_OPT_WAVE)
+    const uint32_t SG = (h->S + 31) / 32;
+    const uint32_t gw = (h->mode == PPR_MODE_SHARED && h->wave) ? h->wave / 32 : SG;
+    for (uint32_t g0 = 0; g0 < SG; g0 += gw) {
+        a.g_lo = gw == SG ? 0u : g0;
+        a.g_hi = gw == SG ? 0u : std::min(SG, g0 + gw);
+        cudaError_t e = u3 ? launch_push_u3(h->mode, a, h->num_sms, h->st)
+                           : launch_push(h->mode, a, h->num_sms, h->st);
+        if (e != cudaSuccess) return cuda_fail(h, e, "push launch");
+        ++*launches;
+    }
     return PPR_OK;
 }
 
@@ -502,8 +565,7 @@ ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
 // restore, push.
 // PPR_DEBUG=1: report the first launch error of a batch with the step that raised it
 inline void dbg_step(const char* what) {
-    static const bool on = getenv("PPR_DEBUG") && atoi(getenv("PPR_DEBUG")) > 0;
-    if (!on) return;
+    if (!dbg_on()) return;
     cudaError_t e = cudaPeekAtLastError();
     if (e != cudaSuccess) fprintf(stderr, "PPR_DEBUG: %s: %s\n", what, cudaGetErrorString(e));
 }
@@ -546,8 +608,8 @@ ppr_status enqueue_batch(ppr_ctx* h, const uint32_t* is, const uint32_t* id, uin
     launch_store_apply(dg, kv, N, b, h->d_ctl, st, &launches);
     dbg_step("launch_store_apply");
     StoreParams sp{h->slack, h->min_cap, h->pool_cap[h->active ^ 1u]};
-    launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches);
-    dbg_step("launch_store_rebuild");
+    const cudaError_t erb = launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches);
+    if (erb != cudaSuccess) return cuda_fail(h, erb, "store rebuild launch");
     launch_seg_cleanup(kv, N, b, h->vb, h->d_ctl, st, &launches);
     dbg_step("launch_seg_cleanup");
     // a2: restore (after validation)
@@ -611,9 +673,11 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     o.slack = 0.25;
     o.min_cap = 4;
     o.relabel = -1;
+    o.layout = PPR_LAYOUT_ARRAYS;
+    o.l2_persist = -1;
     if (opts) o = *opts;
     if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_SORTAGG || !(o.slack >= 0.0) ||
-        o.min_cap == 0)
+        o.min_cap == 0 || (o.layout != PPR_LAYOUT_ARRAYS && o.layout != PPR_LAYOUT_PACKED))
         return PPR_EINVAL;
 
     ppr_ctx* h = new (std::nothrow) ppr_ctx();
@@ -650,13 +714,9 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     cudaEventCreateWithFlags(&h->ev_valid, cudaEventDisableTiming);
     cudaEventCreateWithFlags(&h->ev_join, cudaEventDisableTiming);
     h->npasses = key_shifts(ceil_log2(h->n), h->shifts);
-    if (getenv("PPR_GRAPHS") && !strcmp(getenv("PPR_GRAPHS"), "0")) h->graphs = false;
-    {   // hybrid tail: PPR_HYBRID=<entries>, 0 = off; the ring
-        // costs 16 B per (source, vertex), so it is only used up to 2^27 of them
-        const char* hy = getenv("PPR_HYBRID");
-        const long long t = hy ? atoll(hy) : 16384;
-        h->hyb_thresh = (t > 0 && (uint64_t)h->S * h->n <= (1ull << 27)) ? (uint64_t)t : 0;
-    }
+    // hybrid tail (PPR_OPT_RING_TAIL): the ring costs
+    // 16 B per (source, vertex), so it is only used up to 2^27 of them
+    h->hyb_thresh = ring_fits(h) ? kRingTailDefault : 0;
     if (getenv("PPR_TRACE") && atoi(getenv("PPR_TRACE")) > 0) {
         h->trace_cap = 4096;
         dalloc(h, &h->d_trace, 4ull * h->trace_cap + 8);
@@ -668,9 +728,14 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     // pools fit 32-bit offsets; arrays (R, P as [S][n]) otherwise
     const double pool_bound = (1.0 + h->slack) * (double)arcs_in * 1.25 + 8.0 * h->n + 4096;
     // Default: arrays (R + d_out = 12 B/vertex stay L2-resident, see ppr_internal.cuh);
-    // PPR_LAYOUT=packed selects the 32-byte records for experiments.
-    const char* lay = getenv("PPR_LAYOUT");
-    const bool packed = lay && !strcmp(lay, "packed") && h->S == 1 && o.mode != PPR_MODE_SHARED && o.mode != PPR_MODE_SORTAGG && pool_bound < 4.0e9;
+    // ppr_opts.layout = PPR_LAYOUT_PACKED selects the 32-byte records (measured slower).
+    if (o.layout == PPR_LAYOUT_PACKED &&
+        !(h->S == 1 && o.mode != PPR_MODE_SHARED && o.mode != PPR_MODE_SORTAGG && pool_bound < 4.0e9)) {
+        destroy_all(h);
+        delete h;
+        return PPR_EINVAL;
+    }
+    const bool packed = o.layout == PPR_LAYOUT_PACKED;
     bool ok = packed ? dalloc(h, &h->d_rec, h->n) == cudaSuccess
                      : (dalloc(h, &h->d_hot, Sn + (h->n + 1) / 2 + 32) == cudaSuccess &&
                         dalloc(h, &h->d_slab, h->n) == cudaSuccess &&
@@ -685,35 +750,22 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         // 37 MB of 79 MB): a window over a larger set (Twitter 480 MB) persists a
         // random hitRatio share of its lines and slows the push by 18%
         // (profiles/round1_l2win.md).  PPR_L2_PERSIST=0 / 1 forces it off / on.
-        const char* pe = getenv("PPR_L2_PERSIST");
         int maxp = 0, maxw = 0;
         cudaDeviceGetAttribute(&maxp, cudaDevAttrMaxPersistingL2CacheSize, h->device);
         cudaDeviceGetAttribute(&maxw, cudaDevAttrMaxAccessPolicyWindowSize, h->device);
-        const bool want = pe ? strcmp(pe, "0") != 0 : h->hot_bytes <= (uint64_t)maxp;
-        if (want) {
-            if (maxp > 0 && maxw > 0) {
-                size_t win = std::min<size_t>(h->hot_bytes, (size_t)maxw);
-                const char* wm = getenv("PPR_L2_WIN_MB");  // experiment: cap the window (hub prefix of R)
-                if (wm && atof(wm) > 0) win = std::min<size_t>(win, (size_t)(atof(wm) * 1048576.0));
-                const size_t setaside = std::min<size_t>(win, (size_t)maxp);
-                size_t cur = 0;
-                cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize);
-                if (cur < setaside) cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, setaside);
-                cudaStreamAttrValue av{};
-                av.accessPolicyWindow.base_ptr = h->d_hot;
-                av.accessPolicyWindow.num_bytes = win;
-                av.accessPolicyWindow.hitRatio = (float)std::min(1.0, (double)setaside / (double)win);
-                av.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
-                av.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
-                h->l2_window =
-                    cudaStreamSetAttribute(h->st, cudaStreamAttributeAccessPolicyWindow, &av) == cudaSuccess;
-                h->l2_win_bytes = win;
-                h->l2_hit = av.accessPolicyWindow.hitRatio;
-                if (getenv("PPR_DEBUG"))
-                    fprintf(stderr, "ppr: L2 window %zu B of %llu hot (max window %d, max set-aside %d), hit ratio %.3f\n",
-                            win, (unsigned long long)h->hot_bytes, maxw, maxp, h->l2_hit);
-                cudaGetLastError();
-            }
+        const bool want = o.l2_persist > 0 || (o.l2_persist < 0 && h->hot_bytes <= (uint64_t)maxp);
+        if (want && maxp > 0 && maxw > 0) {
+            // the window travels with each push launch (launch attribute); the
+            // caller's stream is left alone.  The device-wide set-aside is raised
+            // while any handle on the device needs it (l2_acquire / l2_release).
+            const size_t win = std::min<size_t>(h->hot_bytes, (size_t)maxw);
+            const size_t setaside = std::min<size_t>(win, (size_t)maxp);
+            h->l2_window = l2_acquire(h->device, setaside);
+            h->l2_win_bytes = h->l2_window ? win : 0;
+            h->l2_hit = (float)std::min(1.0, (double)setaside / (double)win);
+            if (dbg_on())
+                fprintf(stderr, "ppr: L2 window %zu B of %llu hot (max window %d, max set-aside %d), hit ratio %.3f\n",
+                        win, (unsigned long long)h->hot_bytes, maxw, maxp, h->l2_hit);
         }
     }
     ok = ok &&
@@ -907,6 +959,23 @@ ppr_status ppr_set_option(ppr_ctx* h, int key, int64_t value) {
             return PPR_OK;
         case PPR_OPT_TIMING: h->timing = value != 0; return PPR_OK;
         case PPR_OPT_FORCE_REBUILD: h->force_rebuild = value != 0; return PPR_OK;
+        case PPR_OPT_RING_TAIL:
+            if (value < 0) return PPR_EINVAL;
+            h->hyb_thresh = (value > 0 && ring_fits(h)) ? (uint64_t)value : 0;
+            return PPR_OK;
+        case PPR_OPT_RING_ALL:
+            if (value < -1 || value > 1) return PPR_EINVAL;
+            h->ring_all = (int)value;
+            return PPR_OK;
+        case PPR_OPT_EDGE_CHAINS:
+            if (value != 0 && value != 2 && value != 3) return PPR_EINVAL;
+            h->edge_chains = (int)value;
+            return PPR_OK;
+        case PPR_OPT_GRAPHS: h->graphs = value != 0; return PPR_OK;
+        case PPR_OPT_WAVE:
+            if (value < 0 || value % 32 != 0 || value > 0xFFFFFFFFll) return PPR_EINVAL;
+            h->wave = (uint32_t)value;
+            return PPR_OK;
         default: return PPR_EINVAL;
     }
 }
@@ -958,7 +1027,7 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     if (use_graph) {  // one graph per batch shape, replayed
         const GraphKey key{n_ins, n_del, h->push_enabled, h->mode, h->max_iters, h->timing,
                            h->force_rebuild, h->buf_epoch, h->pool_cap[0], h->pool_cap[1],
-                           (const void*)h->d_pool[0], (const void*)h->d_pool[1]};
+                           (const void*)h->d_pool[0], (const void*)h->d_pool[1], h->active};
         if (!h->gexec || !(key == h->gkey)) {
             if (h->gexec) cudaGraphExecDestroy(h->gexec), h->gexec = nullptr;
             cudaGraph_t graph = nullptr;

@@ -54,7 +54,18 @@ struct DevStats {
     unsigned int n_big;        // vertices copied warp-wide in a rebuild
     unsigned int pad0;
     unsigned long long walk_edges; // in-arc walks (SHARED: one per (source group, arc))
+    // device clock (%globaltimer, ns): POS / NEG phase durations summed over the
+    // push launches of a call (one, or one per source wave); restore kernel
+    // first-CTA start (atomicMin) and last-CTA end (atomicMax)
+    unsigned long long ns_push[2];
+    unsigned long long t_restore[2];
 };
+
+__device__ __forceinline__ unsigned long long globaltimer_ns() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+    return t;
+}
 
 // A counter alone on its 128-byte line: the per-round counters, the tile
 // claims and the grid barrier are hammered by every CTA, so none of them

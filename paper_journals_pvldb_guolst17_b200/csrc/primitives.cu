@@ -15,6 +15,10 @@
 // loads are coalesced and the (round, thread) order is the input order,
 // which keeps the sort stable.
 #include "primitives.cuh"
+
+#include <map>
+#include <mutex>
+#include <utility>
 #include "block_scan.cuh"
 
 namespace ppr {
@@ -238,6 +242,32 @@ void exclusive_scan_u32(const uint32_t* in, unsigned long long* out, uint64_t n,
     k_scan_part<<<1, SCAN_THREADS, 0, st>>>(part, np, total);
     k_scan_down<<<(unsigned)np, SCAN_THREADS, 0, st>>>(in, n, part, out);
     *launches += 3;
+}
+
+cudaError_t blocks_per_sm(const void* fn, int threads, int cap, int* out) {
+    static std::mutex mu;
+    static std::map<std::pair<int, const void*>, int> cache;
+    int dev = 0;
+    cudaError_t e = cudaGetDevice(&dev);
+    if (e != cudaSuccess) return e;
+    const auto key = std::make_pair(dev, fn);
+    {
+        std::lock_guard<std::mutex> lk(mu);
+        auto it = cache.find(key);
+        if (it != cache.end()) {
+            *out = it->second;
+            return cudaSuccess;
+        }
+    }
+    int b = 0;
+    e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, fn, threads, 0);
+    if (e != cudaSuccess) return e;
+    if (b < 1) return cudaErrorInvalidConfiguration;
+    if (b > cap) b = cap;
+    std::lock_guard<std::mutex> lk(mu);
+    cache[key] = b;
+    *out = b;
+    return cudaSuccess;
 }
 
 }  // namespace ppr

@@ -45,4 +45,9 @@ void exclusive_scan_u32(const uint32_t* in, unsigned long long* out, uint64_t n,
 // digit shifts for keys (hi << 32 | lo) with hi, lo < 2^bits
 int key_shifts(int bits, int* shifts /* >= 8 */);
 
+// Resident CTAs per SM of kernel `fn` at `threads` threads on the calling
+// thread's current device, capped at `cap`: cached per (device, kernel),
+// thread-safe (persistent and cooperative grids are sized from it).
+cudaError_t blocks_per_sm(const void* fn, int threads, int cap, int* out);
+
 }  // namespace ppr

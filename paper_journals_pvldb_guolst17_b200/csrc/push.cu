@@ -37,6 +37,7 @@
 // full slice is flushed by its warp with one global atomic, and the CTA
 // flushes all slices with one atomic at the end of a round.
 #include "block_scan.cuh"
+#include "primitives.cuh"
 #include "push.cuh"
 
 namespace ppr {
@@ -45,28 +46,18 @@ namespace {
 
 constexpr int PT = PUSH_THREADS;
 constexpr int NW = PT / 32;     // warps per CTA
-#ifndef PPR_PUSH_OVERLAP
-#define PPR_PUSH_OVERLAP 1
-#endif
-#ifndef PPR_PUSH_DYN
-#define PPR_PUSH_DYN 1
-#endif
 #ifndef PPR_PUSH_U
 #define PPR_PUSH_U 2
 #endif
 #ifndef PPR_PUSH_OPT_ONLY
 #define PPR_PUSH_OPT_ONLY 0
 #endif
-// Opt self-update by exchange: r_u = atomicExch(R(u), 0) (DESIGN.md K-PUSH)
 // per-CTA time split of the trace (PPR_TRACE): compiled in only on request,
 // its counters would otherwise cost registers in every thread
 #ifndef PPR_PUSH_TIMESPLIT
 #define PPR_PUSH_TIMESPLIT 0
 #endif
 constexpr bool kTimeSplit = PPR_PUSH_TIMESPLIT;
-#ifndef PPR_PUSH_XCHG
-#define PPR_PUSH_XCHG 1
-#endif
 constexpr int U = PPR_PUSH_U;   // edges per lane per step
 #ifndef PPR_PUSH_QW
 #define PPR_PUSH_QW 256
@@ -79,11 +70,14 @@ enum { K_OPT = 0, K_EAGER = 1, K_DUP = 2, K_VAN = 3, K_SCAN = 4 };
 // fire-and-forget reduction that also marks the touched vertex in a bitmap;
 // the next frontier is decided after a grid barrier by scanning the bitmap.
 
-struct Smem {
+struct TileArrays {
     uint32_t scan[PT + 1];                // exclusive in-degree prefix of the tile
+    uint32_t sid[PT];                     // source index of each entry
     unsigned long long off[PT];           // slab offset of each entry
     double w[PT];                         // (1-a) * r of each entry
-    uint32_t sid[PT];                     // source index of each entry
+};
+struct Smem {
+    TileArrays t;                         // the CTA's current tile
     unsigned long long q[NW][QW];         // per-warp enqueue slices
     unsigned int wq[NW];                  // slice fill at the end-of-round flush
     unsigned long long gbase;
@@ -93,11 +87,6 @@ struct Smem {
     uint32_t warp_tmp[NW + 1];            // block-scan scratch
 };
 
-__device__ __forceinline__ unsigned long long global_ns() {
-    unsigned long long t;
-    asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
-    return t;
-}
 
 struct Ctx {
     const uint32_t* pool;
@@ -221,84 +210,19 @@ __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
     tile_body<POS, KIND, PK>(s, c, a, valid, ent, idx, T, top);
 }
 
-// The tile's work once thread i holds entry i (valid, ent; idx indexes W).
+// Walks the E edges of one prepared tile (scan/off/w/sid, the entries' in-lists
+// concatenated): warps claim U consecutive 32-edge chunks at a time from
+// *chunkp, lane k of a chunk takes edge k, finds its owner entry by binary
+// search in the prefix, and runs the chain pool entry -> d_out(v) ->
+// atomicAdd(R(v), (1-a) r_u / d(v)) (Alg 3 lines 17-20 / Alg 4 lines 11-17).
+// All U atomics of a step are issued before any result is consumed.
 template <bool POS, int KIND, bool PK>
-__device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
-                                          unsigned long long ent, uint64_t idx, uint32_t T,
-                                          int top) {
+__device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, const TileArrays& t,
+                                           uint32_t E, int top, unsigned int* chunkp) {
     const unsigned L = lane(), w = warp();
-    const double eps = a.g.eps, alpha = a.g.alpha;
+    const double eps = a.g.eps;
     const uint32_t n = a.g.n;
-    const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
-    double* ru = Rp<PK>(a.g, sidx, u);
-    double r = 0.0;
-    bool push = false;
-    if (KIND == K_OPT && PPR_PUSH_XCHG) {
-        // Alg 4 lines 10 and 20-21 as one atomic: r_u = R(u), R(u) = 0.  Adds that
-        // reach u before the exchange are absorbed into r_u (P:1102-1112); adds
-        // after it start from 0, so u's next crossing re-enqueues it exactly once.
-        r = valid ? atom_exch_f64_pol(ru, 0.0, l2_keep()) : 0.0;
-        push = valid && r != 0.0;
-        if (push) red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
-    } else if (KIND == K_OPT || KIND == K_EAGER || KIND == K_SCAN) {
-        r = valid ? ld_relaxed_f64(ru) : 0.0;  // Alg 4 line 10: the current R(u)
-        // A queued vertex meets pushCond (it was enqueued on a crossing, and R(u)
-        // only grows until its own self-update).  If the relaxed load returned
-        // an older value (the async schedule has no barrier ordering it after
-        // the enqueuer's atomic), re-read at the coherence point.
-        if (KIND == K_OPT && valid && !push_cond<POS>(r, eps)) r = atomicAdd(ru, 0.0);
-        push = valid && push_cond<POS>(r, eps);
-        if (KIND == K_EAGER && valid) __stcg(&a.W[idx], push ? r : 0.0);
-    } else {
-        r = valid ? __ldcg(&a.W[idx]) : 0.0;   // Alg 3: the snapshot S
-        push = valid;
-    }
-    // Alg 4 lines 20-21, fused and issued before the edge walk so its latency
-    // overlaps it: R(u) -= r_u atomically (its result decides the re-enqueue,
-    // DESIGN.md K-PUSH) and P(u) += a r_u as a fire-and-forget reduction (one
-    // entry per vertex per round, so no contention).
-    double self_old = 0.0;
-    if (KIND == K_OPT && !PPR_PUSH_XCHG && push) {
-        self_old = atomicAdd(ru, -r);
-        red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
-    }
-    if (KIND == K_SCAN && push) {  // self-update: no result needed; u is re-tested at the scan
-        red_add_pol(ru, -r, l2_keep());
-        red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
-        mark_bit(a.bitmap, (size_t)u * a.g.S + sidx);
-        c.pushes++;
-    }
-    uint32_t len = 0;
-    unsigned long long off = 0;
-    if (push) {
-        if (PK) {  // {off, len} of the vertex record (same sector as R(u), P(u))
-            const uint2 q = __ldcg(reinterpret_cast<const uint2*>(&a.g.rec[u].off));
-            off = q.x;
-            len = q.y;
-        } else {
-            const ulonglong2 sl = ld_u64x2_pol(&a.g.slab[u], l2_stream());
-            off = sl.x;               // Slab::off
-            len = (uint32_t)sl.y;     // Slab::len (low word of {len, cap})
-        }
-    }
-    uint32_t E;
-    const uint32_t ex = block_exclusive_scan_u32<PT>(len, s.warp_tmp, &E);
-    s.scan[threadIdx.x] = threadIdx.x < T ? ex : 0xFFFFFFFFu;
-    if (threadIdx.x == 0) {
-        s.scan[PT] = 0xFFFFFFFFu;
-        s.chunk = 0;
-    }
-    s.off[threadIdx.x] = off;
-    s.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
-    s.sid[threadIdx.x] = sidx;
-    __syncthreads();
-    if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_pro += global_ns() - c.t_mark;
-    if (threadIdx.x == 0) {
-        c.edges += E;
-        if (c.trace_edges && E) atomicAdd(c.trace_edges, (unsigned long long)E);
-    }
     const unsigned long long pol_keep = l2_keep(), pol_stream = l2_stream();
-    // 32-edge chunks dealt round-robin to the warps (chunk w + NW*i), U per step
     if constexpr (KIND == K_SCAN) {  // fire-and-forget edge walk: no enqueue decisions here
         for (uint32_t cb = w; cb * 32 < E; cb += NW * U) {
             uint32_t v[U], d[U];
@@ -309,8 +233,8 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
                 j[k] = -1;
                 v[k] = 0;
                 if (e < E) {
-                    j[k] = owner_of(s.scan, e, top);
-                    v[k] = ld_pool(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
+                    j[k] = owner_of(t.scan, e, top);
+                    v[k] = ld_pool(&c.pool[t.off[j[k]] + (e - t.scan[j[k]])], pol_stream);
                 }
             }
 #pragma unroll
@@ -319,53 +243,44 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
 #pragma unroll
             for (int k = 0; k < U; k++) {
                 if (j[k] >= 0) {
-                    const uint32_t sj = s.sid[j[k]];
-                    red_add_pol(Rp<PK>(a.g, sj, v[k]), __ddiv_rn(s.w[j[k]], (double)d[k]), pol_keep);
+                    const uint32_t sj = t.sid[j[k]];
+                    red_add_pol(Rp<PK>(a.g, sj, v[k]), __ddiv_rn(t.w[j[k]], (double)d[k]), pol_keep);
                     mark_bit(a.bitmap, (size_t)v[k] * a.g.S + sj);
                 }
             }
         }
     } else {
-#if PPR_PUSH_DYN
     // warps claim U consecutive 32-edge chunks at a time from a shared counter,
-    // so a warp whose atomics return late does not hold the tile's barrier
+    // so a warp whose atomics return late does not hold up the others
     while (true) {
         uint32_t cb = 0;
-        if (L == 0) cb = atomicAdd(&s.chunk, (unsigned)U);
+        if (L == 0) cb = atomicAdd(chunkp, (unsigned)U);
         cb = __shfl_sync(0xffffffffu, cb, 0);
         if (cb * 32 >= E) break;
-#define PPR_CHUNK(k) (cb + (k))
-#else
-    for (uint32_t cb = w; cb * 32 < E; cb += NW * U) {
-#define PPR_CHUNK(k) (cb + NW * (k))
-#endif
         ensure_room(s, c, 32 * U);
         uint32_t v[U];
         int j[U];
 #pragma unroll
         for (int k = 0; k < U; k++) {
-            const uint32_t e = PPR_CHUNK(k) * 32 + L;
+            const uint32_t e = (cb + k) * 32 + L;
             j[k] = -1;
             v[k] = 0;
             if (e < E) {
-                j[k] = owner_of(s.scan, e, top);
-                v[k] = ld_pool(&c.pool[s.off[j[k]] + (e - s.scan[j[k]])], pol_stream);
+                j[k] = owner_of(t.scan, e, top);
+                v[k] = ld_pool(&c.pool[t.off[j[k]] + (e - t.scan[j[k]])], pol_stream);
             }
         }
         uint32_t d[U];
 #pragma unroll
         for (int k = 0; k < U; k++)
             d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_dout(&a.g.dout[v[k]], pol_keep));
-#if PPR_PUSH_OVERLAP
-        // all U atomics are issued before any result is consumed, so the U
-        // chains overlap (the enqueues below synchronise the warp)
         double incr[U], pre[U];
         uint32_t sj[U];
 #pragma unroll
         for (int k = 0; k < U; k++) {
             if (j[k] >= 0) {
-                sj[k] = s.sid[j[k]];
-                incr[k] = __ddiv_rn(s.w[j[k]], (double)d[k]);
+                sj[k] = t.sid[j[k]];
+                incr[k] = __ddiv_rn(t.w[j[k]], (double)d[k]);
                 pre[k] = atom_add_pol(Rp<PK>(a.g, sj[k], v[k]), incr[k], pol_keep);
             }
         }
@@ -384,39 +299,77 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             }
             warp_enqueue(s, c, enq, ev);
         }
-#else
-#pragma unroll
-        for (int k = 0; k < U; k++) {
-            bool enq = false;
-            unsigned long long ev = 0;
-            if (j[k] >= 0) {
-                const uint32_t sj = s.sid[j[k]];
-                const double incr = __ddiv_rn(s.w[j[k]], (double)d[k]);
-                const double pre = atom_add_pol(Rp<PK>(a.g, sj, v[k]), incr, pol_keep);
-                const double cur = __dadd_rn(pre, incr);  // == the stored value (no FMA)
-                ev = ((unsigned long long)sj << 32) | v[k];
-                if (KIND == K_OPT || KIND == K_DUP)
-                    enq = crossed<POS>(pre, cur, eps);   // Alg 4 line 16
-                else
-                    enq = push_cond<POS>(cur, eps) &&
-                          test_and_set(a.bitmap, (size_t)sj * n + v[k]);  // UniqueEnqueue
-            }
-            warp_enqueue(s, c, enq, ev);
-        }
-#endif
-    }
-    if (KIND == K_OPT && PPR_PUSH_XCHG) {
-        if (push) c.pushes++;
-    } else if (KIND == K_OPT) {  // re-enqueue on the result of the fused self-update
-        bool re = false;
-        if (push) {
-            re = push_cond<POS>(__dadd_rn(self_old, -r), eps);
-            c.pushes++;
-        }
-        ensure_room(s, c, 32);
-        warp_enqueue(s, c, re, ent);
     }
     }  // not K_SCAN
+}
+
+// The tile's work once thread i holds entry i (valid, ent; idx indexes W):
+// the entry's residual read / self-update, the CTA-wide prefix of the
+// pushed entries' in-degrees, then the edge walk by all warps.
+template <bool POS, int KIND, bool PK>
+__device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
+                                          unsigned long long ent, uint64_t idx, uint32_t T,
+                                          int top) {
+    const double eps = a.g.eps, alpha = a.g.alpha;
+    const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
+    double* ru = Rp<PK>(a.g, sidx, u);
+    double r = 0.0;
+    bool push = false;
+    // the slab descriptor depends only on u: issued before (and overlapping)
+    // the residual read below, used only if the entry pushes
+    uint32_t len = 0;
+    unsigned long long off = 0;
+    if (valid) {
+        if (PK) {  // {off, len} of the vertex record (same sector as R(u), P(u))
+            const uint2 q = __ldcg(reinterpret_cast<const uint2*>(&a.g.rec[u].off));
+            off = q.x;
+            len = q.y;
+        } else {
+            const ulonglong2 sl = ld_u64x2_pol(&a.g.slab[u], l2_stream());
+            off = sl.x;               // Slab::off
+            len = (uint32_t)sl.y;     // Slab::len (low word of {len, cap})
+        }
+    }
+    if (KIND == K_OPT) {
+        // Alg 4 lines 10 and 20-21 as one atomic: r_u = R(u), R(u) = 0.  Adds that
+        // reach u before the exchange are absorbed into r_u (P:1102-1112); adds
+        // after it start from 0, so u's next crossing re-enqueues it exactly once
+        // (DESIGN.md K-PUSH).
+        r = valid ? atom_exch_f64_pol(ru, 0.0, l2_keep()) : 0.0;
+        push = valid && r != 0.0;
+        if (push) red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
+    } else if (KIND == K_EAGER || KIND == K_SCAN) {
+        r = valid ? ld_relaxed_f64(ru) : 0.0;  // Alg 4 line 10: the current R(u)
+        push = valid && push_cond<POS>(r, eps);
+        if (KIND == K_EAGER && valid) __stcg(&a.W[idx], push ? r : 0.0);
+    } else {
+        r = valid ? __ldcg(&a.W[idx]) : 0.0;   // Alg 3: the snapshot S
+        push = valid;
+    }
+    if (KIND == K_SCAN && push) {  // self-update: no result needed; u is re-tested at the scan
+        red_add_pol(ru, -r, l2_keep());
+        red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
+        mark_bit(a.bitmap, (size_t)u * a.g.S + sidx);
+    }
+    if (!push) len = 0;
+    if (push && KIND != K_VAN && KIND != K_DUP && KIND != K_EAGER) c.pushes++;
+    uint32_t E;
+    const uint32_t ex = block_exclusive_scan_u32<PT>(len, s.warp_tmp, &E);
+    s.t.scan[threadIdx.x] = threadIdx.x < T ? ex : 0xFFFFFFFFu;
+    if (threadIdx.x == 0) {
+        s.t.scan[PT] = 0xFFFFFFFFu;
+        s.chunk = 0;
+    }
+    s.t.off[threadIdx.x] = off;
+    s.t.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
+    s.t.sid[threadIdx.x] = sidx;
+    __syncthreads();
+    if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_pro += globaltimer_ns() - c.t_mark;
+    if (threadIdx.x == 0) {
+        c.edges += E;
+        if (c.trace_edges && E) atomicAdd(c.trace_edges, (unsigned long long)E);
+    }
+    walk_edges<POS, KIND, PK>(s, c, a, s.t, E, top, &s.chunk);
 }
 
 // Every CTA takes tiles of T entries: its first tile statically, the rest by
@@ -433,17 +386,18 @@ __device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a
     const uint64_t ntiles = (C + T - 1) / T;
     uint64_t t = blockIdx.x;
     while (t < ntiles) {
-        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark = global_ns();
+        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark = globaltimer_ns();
         cta_tile<POS, KIND, PK>(s, c, a, Fin, C, t * T, T, top);
-        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark2 = global_ns();
+        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark2 = globaltimer_ns();
         if (ntiles <= gridDim.x) break;  // every tile was assigned statically
         if (threadIdx.x == 0) s.next = atomicAdd(tc, 1ull) + gridDim.x;
         __syncthreads();
         t = s.next;
         __syncthreads();
-        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_claim += global_ns() - c.t_mark2;
+        if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_claim += globaltimer_ns() - c.t_mark2;
     }
 }
+
 
 // ---------------------------------------------------------------- Alg 3 / Eager sessions
 
@@ -636,7 +590,7 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
         if (blockIdx.x == 0 && threadIdx.x == 0) {
             if (c.trace_edges) {
                 a.trace[4ull * it] = C | ((unsigned long long)ph << 63);
-                a.trace[4ull * it + 1] = global_ns();
+                a.trace[4ull * it + 1] = globaltimer_ns();
             }
             ctl->fcount[(it + 2) % 3].v = 0;
             ctl->tilectr[(it + 2) % 3].v = 0;
@@ -660,7 +614,7 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
         c.Fout = a.F[(it + 1) & 1];
         c.cnt_out = &ctl->fcount[(it + 1) % 3].v;
         unsigned long long* tc = &ctl->tilectr[it % 3].v;
-        const unsigned long long t0 = (kTimeSplit && a.trace) ? global_ns() : 0;
+        const unsigned long long t0 = (kTimeSplit && a.trace) ? globaltimer_ns() : 0;
         if (MODE == M_OPT) {
             propagate_all<POS, K_OPT, PK>(s, c, a, Fin, C, tc);
         } else if (MODE == M_SCAN) {
@@ -681,12 +635,12 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
             grid_sync(ctl);
             session_eager_self<POS, PK>(s, c, a, Fin, C);
         }
-        const unsigned long long t1 = (kTimeSplit && a.trace) ? global_ns() : 0;
+        const unsigned long long t1 = (kTimeSplit && a.trace) ? globaltimer_ns() : 0;
         block_flush(s, c);
-        const unsigned long long t2 = (kTimeSplit && a.trace) ? global_ns() : 0;
+        const unsigned long long t2 = (kTimeSplit && a.trace) ? globaltimer_ns() : 0;
         grid_sync(ctl);
         if (kTimeSplit && a.trace) {
-            const unsigned long long t3 = global_ns();
+            const unsigned long long t3 = globaltimer_ns();
             c.t_work += t1 - t0;
             c.t_flush += t2 - t1;
             c.t_bar += t3 - t2;
@@ -723,12 +677,19 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
         for (int i = 0; i < 3; i++) a.ctl->fcount[i].v = a.ctl->tilectr[i].v = 0;
     }
     grid_sync(a.ctl);
+    const bool stamp = blockIdx.x == 0 && threadIdx.x == 0;
+    const unsigned long long t0 = stamp ? globaltimer_ns() : 0;
     unsigned it = 0;
     if (a.phases & 1) run_phase<MODE, true, PK>(s, c, a, it);
+    const unsigned long long t1 = stamp ? globaltimer_ns() : 0;  // run_phase ends with a grid barrier
     if (a.phases & 2) run_phase<MODE, false, PK>(s, c, a, it);
+    if (stamp) {  // phase durations, summed over launches (source waves)
+        atomicAdd(&a.ctl->st.ns_push[0], t1 - t0);
+        atomicAdd(&a.ctl->st.ns_push[1], globaltimer_ns() - t1);
+    }
     if (a.trace && blockIdx.x == 0 && threadIdx.x == 0 && it < a.trace_cap) {
         a.trace[4ull * it] = ~0ull;  // end marker
-        a.trace[4ull * it + 1] = global_ns();
+        a.trace[4ull * it + 1] = globaltimer_ns();
     }
     if (kTimeSplit && a.trace && threadIdx.x == 0) {  // per-CTA time split, summed over CTAs
         atomicAdd(&a.trace[4ull * a.trace_cap + 0], c.t_work);
@@ -825,8 +786,10 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
                         continue;
                     }
                 }
-                const unsigned long long d = *(volatile unsigned long long*)done;
-                const unsigned long long t2 = *(volatile unsigned long long*)tail;
+                // acquire: a `done` that counts an entry makes that entry's
+                // children (added to `tail` before it, released below) visible
+                const unsigned long long d = ld_acquire_u64(done);
+                const unsigned long long t2 = ld_acquire_u64(tail);
                 if (d == t2) {
                     flag = 1;
                     break;
@@ -855,7 +818,10 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
         while (top * 2 < (int)k) top <<= 1;
         tile_body<POS, K_OPT, PK>(s, c, a, valid, ent, 0, k, top);
         block_flush(s, c);  // this tile's children reach `tail` ...
-        if (threadIdx.x == 0) atomicAdd(done, (unsigned long long)k);  // ... before it counts as done
+        if (threadIdx.x == 0) {  // ... before it counts as done (release: tail and the slots first)
+            __threadfence();
+            atomicAdd(done, (unsigned long long)k);
+        }
     }
 }
 
@@ -898,8 +864,15 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid
         for (int i = 0; i < 3; i++) a.ctl->fcount[i].v = a.ctl->tilectr[i].v = 0;
     }
     grid_sync(a.ctl);
+    const bool stamp = blockIdx.x == 0 && threadIdx.x == 0;
+    const unsigned long long t0 = stamp ? globaltimer_ns() : 0;
     if (a.phases & 1) async_phase<true, PK>(s, c, a);
+    const unsigned long long t1 = stamp ? globaltimer_ns() : 0;  // async_phase ends with a grid barrier
     if (a.phases & 2) async_phase<false, PK>(s, c, a);
+    if (stamp) {  // phase durations, summed over launches (source waves)
+        atomicAdd(&a.ctl->st.ns_push[0], t1 - t0);
+        atomicAdd(&a.ctl->st.ns_push[1], globaltimer_ns() - t1);
+    }
     __shared__ unsigned long long s_red[2];
     if (threadIdx.x == 0) s_red[0] = s_red[1] = 0;
     __syncthreads();
@@ -914,28 +887,18 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid
 
 template <bool PK>
 cudaError_t launch_async(const PushArgs& a, int num_sms, cudaStream_t st) {
-    static int blocks_per_sm = 0;
-    if (blocks_per_sm == 0) {
-        cudaError_t e =
-            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push_async<PK>, PT, 0);
-        if (e != cudaSuccess) return e;
-        if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
-        if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
-    }
-    return coop_launch((const void*)k_push_async<PK>, num_sms * blocks_per_sm, a, st);
+    int bps = 0;
+    const cudaError_t e = blocks_per_sm((const void*)k_push_async<PK>, PT, PUSH_MIN_BLOCKS, &bps);
+    if (e != cudaSuccess) return e;
+    return coop_launch((const void*)k_push_async<PK>, num_sms * bps, a, st);
 }
 
 template <int MODE, bool PK>
 cudaError_t launch_mode(const PushArgs& a, int num_sms, cudaStream_t st) {
-    static int blocks_per_sm = 0;
-    if (blocks_per_sm == 0) {
-        cudaError_t e =
-            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push<MODE, PK>, PT, 0);
-        if (e != cudaSuccess) return e;
-        if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
-        if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
-    }
-    return coop_launch((const void*)k_push<MODE, PK>, num_sms * blocks_per_sm, a, st);
+    int bps = 0;
+    const cudaError_t e = blocks_per_sm((const void*)k_push<MODE, PK>, PT, PUSH_MIN_BLOCKS, &bps);
+    if (e != cudaSuccess) return e;
+    return coop_launch((const void*)k_push<MODE, PK>, num_sms * bps, a, st);
 }
 
 template <bool PK>

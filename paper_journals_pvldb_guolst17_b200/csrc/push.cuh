@@ -38,6 +38,7 @@ struct PushArgs {
     unsigned long long ring_cap;
     int hyb_all;               // Opt: every phase runs on the ring from its seeds (dense graphs)
     uint64_t hyb_thresh;       // Opt: a phase whose frontier is <= this many entries finishes on the ring (0: off)
+    uint32_t g_lo, g_hi;       // SHARED: source groups [g_lo, g_hi) of this launch (a wave); 0, 0: all
     unsigned long long* trace; // optional: 4 words per round {C | phase<<63, t_ns, edges, -}
     uint32_t trace_cap;        // rounds the trace buffer holds
 };

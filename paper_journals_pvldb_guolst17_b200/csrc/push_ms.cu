@@ -33,6 +33,7 @@
 // divides, the two differ by at most one rounding per increment, far inside
 // the invariant tolerance R18).
 #include "block_scan.cuh"
+#include "primitives.cuh"
 #include "push.cuh"
 
 namespace ppr {
@@ -363,24 +364,32 @@ __device__ __forceinline__ void ms_scan(MsSmem& s, MsCtx& c, const PushArgs& a, 
     }
 }
 
-// marks the phase's seeds
+// marks the phase's seeds: every (seed vertex, group) of the launch's group
+// range [g0, g1) (all groups, or one wave of them)
 __device__ __forceinline__ void ms_seed(const PushArgs& a, uint32_t SG) {
     const uint64_t stride = (uint64_t)gridDim.x * PT;
     const uint64_t t0 = (uint64_t)blockIdx.x * PT + threadIdx.x;
+    const uint32_t g0 = a.g_hi ? a.g_lo : 0u, g1 = a.g_hi ? a.g_hi : SG, G = g1 - g0;
     if (a.seed_all) {
-        const uint64_t nbits = (uint64_t)SG * a.g.n, nwords = (nbits + 31) / 32;
-        for (uint64_t wi = t0; wi < nwords; wi += stride) {
-            const uint64_t rem = nbits - wi * 32;
-            a.bitmap[wi] = rem >= 32 ? 0xFFFFFFFFu : ((1u << rem) - 1u);
+        if (G == SG) {
+            const uint64_t nbits = (uint64_t)SG * a.g.n, nwords = (nbits + 31) / 32;
+            for (uint64_t wi = t0; wi < nwords; wi += stride) {
+                const uint64_t rem = nbits - wi * 32;
+                a.bitmap[wi] = rem >= 32 ? 0xFFFFFFFFu : ((1u << rem) - 1u);
+            }
+        } else {
+            for (uint64_t k = t0; k < (uint64_t)a.g.n * G; k += stride)
+                mark(a.bitmap, (k / G) * SG + g0 + k % G);
         }
     } else if (a.seed_v) {
         const uint64_t nv = *a.n_seed_v_dev;
-        for (uint64_t k = t0; k < nv * SG; k += stride)
-            mark(a.bitmap, (unsigned long long)a.seed_v[k / SG] * SG + (k % SG));
+        for (uint64_t k = t0; k < nv * G; k += stride)
+            mark(a.bitmap, (unsigned long long)a.seed_v[k / G] * SG + g0 + (k % G));
     } else {
         for (uint64_t k = t0; k < a.n_seed_e; k += stride) {
             const unsigned long long ent = a.seed_e[k];
-            mark(a.bitmap, (unsigned long long)(uint32_t)ent * SG + (uint32_t)(ent >> 32) / 32);
+            const uint32_t g = (uint32_t)(ent >> 32) / 32;
+            if (g >= g0 && g < g1) mark(a.bitmap, (unsigned long long)(uint32_t)ent * SG + g);
         }
     }
 }
@@ -446,9 +455,16 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_co
     if (blockIdx.x == 0 && threadIdx.x == 0)
         for (int i = 0; i < 3; i++) a.ctl->fcount[i].v = a.ctl->tilectr[i].v = 0;
     grid_sync(a.ctl);
+    const bool stamp = blockIdx.x == 0 && threadIdx.x == 0;
+    const unsigned long long t0 = stamp ? globaltimer_ns() : 0;
     unsigned it = 0;
     if (a.phases & 1) ms_phase<true>(s, c, a, SG, it);
+    const unsigned long long t1 = stamp ? globaltimer_ns() : 0;  // ms_phase ends with a grid barrier
     if (a.phases & 2) ms_phase<false>(s, c, a, SG, it);
+    if (stamp) {  // phase durations, summed over launches (source waves)
+        atomicAdd(&a.ctl->st.ns_push[0], t1 - t0);
+        atomicAdd(&a.ctl->st.ns_push[1], globaltimer_ns() - t1);
+    }
     __shared__ unsigned long long s_red[3];
     if (threadIdx.x < 3) s_red[threadIdx.x] = 0;
     __syncthreads();
@@ -466,17 +482,13 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_co
 }  // namespace
 
 cudaError_t launch_push_ms(const PushArgs& a, int num_sms, cudaStream_t st) {
-    static int blocks_per_sm = 0;
-    if (blocks_per_sm == 0) {
-        cudaError_t e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks_per_sm, k_push_ms, PT, 0);
-        if (e != cudaSuccess) return e;
-        if (blocks_per_sm < 1) return cudaErrorInvalidConfiguration;
-        if (blocks_per_sm > PUSH_MIN_BLOCKS) blocks_per_sm = PUSH_MIN_BLOCKS;
-    }
+    int bps = 0;
+    const cudaError_t e = blocks_per_sm((const void*)k_push_ms, PT, PUSH_MIN_BLOCKS, &bps);
+    if (e != cudaSuccess) return e;
     PushArgs copy = a;
     void* args[] = {&copy};
     cudaLaunchConfig_t cfg{};
-    cfg.gridDim = dim3(num_sms * blocks_per_sm);
+    cfg.gridDim = dim3(num_sms * bps);
     cfg.blockDim = dim3(PT);
     cfg.stream = st;
     cudaLaunchAttribute at[2];

@@ -99,6 +99,9 @@ __global__ void k_ctl_reset(DevCtl* ctl) {
     ctl->st.n_vheads = ctl->st.n_uheads = ctl->st.n_touched = 0;
     ctl->st.arc_delta = 0;
     ctl->st.n_big = 0;
+    ctl->st.ns_push[0] = ctl->st.ns_push[1] = 0;
+    ctl->st.t_restore[0] = ~0ull;
+    ctl->st.t_restore[1] = 0;
 }
 
 __global__ void k_batch_keys(const uint32_t* __restrict__ is, const uint32_t* __restrict__ id,
@@ -449,6 +452,7 @@ template <bool PK>
 __global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t N, BatchBufs b,
                           uint32_t* __restrict__ touched, DevCtl* ctl) {
     if (*(volatile int*)&ctl->st.err != KERR_OK) return;
+    if (threadIdx.x == 0) atomicMin(&ctl->st.t_restore[0], globaltimer_ns());
     const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_uheads;
     const double a = g.alpha;
     for (uint64_t k = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; k < nseg;
@@ -489,6 +493,8 @@ __global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t 
         const unsigned pos = atomicAdd(&ctl->st.n_touched, 1u);
         touched[pos] = u;
     }
+    __syncthreads();
+    if (threadIdx.x == 0) atomicMax(&ctl->st.t_restore[1], globaltimer_ns());
 }
 
 // ---------------------------------------------------------------- build / init / export
@@ -601,7 +607,7 @@ __global__ void k_degree_keys(const uint32_t* __restrict__ deg, uint32_t n, uint
     }
 }
 
-// spread = k > 0 (default 1; PPR_RELABEL_SPREAD): inside every full block of
+// spread = k > 0 (1 is used): inside every full block of
 // 16 L ranks (L = 16^k lines of 16 residuals) rank i goes to line i % L, slot
 // i / L, so consecutive (equally hot) ranks land on different 128-byte residual
 // lines -- and L2 slices -- while the block's footprint stays L lines (measured:
@@ -707,18 +713,17 @@ void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const
     ++*launches;
 }
 
-void launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
-                          const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
-                          cudaStream_t st, uint32_t* launches) {
+cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
+                                 const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
+                                 cudaStream_t st, uint32_t* launches) {
     (void)N;
-    static int grid = 0;
-    if (grid == 0) {
-        int per_sm = 0, sms = 0, dev = 0;
-        cudaGetDevice(&dev);
-        cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_rebuild<false>, RB_THREADS, 0);
-        grid = sms * (per_sm < 4 ? (per_sm < 1 ? 1 : per_sm) : 4);
-    }
+    const void* fn = g.rec ? (const void*)k_rebuild<true> : (const void*)k_rebuild<false>;
+    int per_sm = 0, sms = 0, dev = 0;
+    cudaError_t e = cudaGetDevice(&dev);
+    if (e == cudaSuccess) e = cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+    if (e == cudaSuccess) e = blocks_per_sm(fn, RB_THREADS, 4, &per_sm);
+    if (e != cudaSuccess) return e;
+    const int grid = sms * per_sm;
     DevGraph gg = g;
     const uint64_t* kk = kv;
     BatchBufs bb = b;
@@ -728,9 +733,9 @@ void launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, con
     uint64_t alt_cap = sp.alt_cap;
     DevCtl* c = ctl;
     void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &alt_cap, &c};
-    const void* fn = g.rec ? (const void*)k_rebuild<true> : (const void*)k_rebuild<false>;
-    cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(RB_THREADS), args, 0, st);
+    e = cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(RB_THREADS), args, 0, st);
     ++*launches;
+    return e;
 }
 
 void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, const VertexBufs& vb,
@@ -801,8 +806,7 @@ void launch_relabel(const uint32_t* src, const uint32_t* dst, uint64_t m, int un
     for (int s = 0; s < lg; s += 8) shifts[np++] = s;
     for (int s = 32; s < 64; s += 8) shifts[np++] = s;
     const int w = radix_sort_pairs(k0, v0, k1, v1, n, shifts, np, hist, st, launches);
-    const char* sp = getenv("PPR_RELABEL_SPREAD");
-    const int spread = sp ? std::max(0, std::min(3, atoi(sp))) : 1;
+    const int spread = 1;  // measured best of 0..3 (round 1)
     k_perm_from_sorted<<<grid_for(n, 256), 256, 0, st>>>(w ? k1 : k0, n, perm, inv, spread);
     *launches += 3;
 }

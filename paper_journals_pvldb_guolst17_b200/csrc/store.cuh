@@ -65,9 +65,9 @@ void launch_store_validate(const DevGraph& g, const uint64_t* kv, uint64_t N, co
 void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                         DevCtl* ctl, cudaStream_t st, uint32_t* launches);
 // a1: sort/merge rebuild into the other pool (skipped unless DevCtl::rebuild)
-void launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
-                          const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
-                          cudaStream_t st, uint32_t* launches);
+cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
+                                 const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
+                                 cudaStream_t st, uint32_t* launches);
 void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, const VertexBufs& vb,
                         DevCtl* ctl, cudaStream_t st, uint32_t* launches);
 

@@ -25,6 +25,8 @@ MODE_OPT, MODE_EAGER, MODE_DUPDETECT, MODE_VANILLA, MODE_ASYNC, MODE_EAGER_SCAN,
 MODES = {"opt": MODE_OPT, "eager": MODE_EAGER, "dupdetect": MODE_DUPDETECT, "vanilla": MODE_VANILLA,
          "async": MODE_ASYNC, "scan": MODE_EAGER_SCAN, "shared": MODE_SHARED, "sortagg": MODE_SORTAGG}
 OPT_MODE, OPT_PUSH, OPT_MAX_ITERS, OPT_TIMING, OPT_FORCE_REBUILD = 1, 2, 3, 4, 5
+OPT_RING_TAIL, OPT_RING_ALL, OPT_EDGE_CHAINS, OPT_GRAPHS, OPT_WAVE = 6, 7, 8, 9, 10
+LAYOUT_ARRAYS, LAYOUT_PACKED = 0, 1
 
 
 class Graph(ctypes.Structure):
@@ -35,7 +37,8 @@ class Graph(ctypes.Structure):
 
 class Opts(ctypes.Structure):
     _fields_ = [("device", ctypes.c_int), ("cuda_stream", ctypes.c_void_p), ("mode", ctypes.c_int),
-                ("slack", ctypes.c_double), ("min_cap", ctypes.c_uint32), ("relabel", ctypes.c_int)]
+                ("slack", ctypes.c_double), ("min_cap", ctypes.c_uint32), ("relabel", ctypes.c_int),
+                ("layout", ctypes.c_int), ("l2_persist", ctypes.c_int)]
 
 
 class BatchStats(ctypes.Structure):
@@ -46,7 +49,8 @@ class BatchStats(ctypes.Structure):
                 ("kernel_launches", ctypes.c_uint32), ("h2d_bytes", ctypes.c_uint64),
                 ("d2h_bytes", ctypes.c_uint64), ("ms_total", ctypes.c_float),
                 ("ms_store", ctypes.c_float), ("ms_restore", ctypes.c_float),
-                ("ms_push", ctypes.c_float), ("walk_edges", ctypes.c_uint64)]
+                ("ms_push", ctypes.c_float), ("walk_edges", ctypes.c_uint64),
+                ("ms_push_pos", ctypes.c_float), ("ms_push_neg", ctypes.c_float)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}
@@ -132,7 +136,8 @@ class Ppr:
     """One PPR handle (one graph, S sources) on one GPU."""
 
     def __init__(self, n, src, dst, sources, alpha=0.15, eps=1e-9, mode="opt", device=0,
-                 stream=None, undirected=False, slack=0.25, min_cap=4, relabel=-1):
+                 stream=None, undirected=False, slack=0.25, min_cap=4, relabel=-1,
+                 layout=LAYOUT_ARRAYS, l2_persist=-1):
         lib = load()
         s, sp = _host_u32(src)
         d, dp = _host_u32(dst)
@@ -141,7 +146,8 @@ class Ppr:
         g = Graph(n=int(n), m=len(s), src=ctypes.cast(sp, ctypes.POINTER(ctypes.c_uint32)),
                   dst=ctypes.cast(dp, ctypes.POINTER(ctypes.c_uint32)), undirected=int(undirected))
         o = Opts(device=int(device), cuda_stream=stream, mode=MODES.get(mode, mode),
-                 slack=float(slack), min_cap=int(min_cap), relabel=int(relabel))
+                 slack=float(slack), min_cap=int(min_cap), relabel=int(relabel),
+                 layout=int(layout), l2_persist=int(l2_persist))
         h = ctypes.c_void_p()
         st = BatchStats()
         rc = lib.ppr_create(ctypes.byref(g), ctypes.cast(sop, ctypes.POINTER(ctypes.c_uint32)),

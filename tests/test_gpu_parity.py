@@ -16,6 +16,7 @@ import oracle
 from oracle import exact
 from paper_journals_pvldb_guolst17_b200 import ppr, workload as W
 from tests import golden_figs as G
+from tests.parity_util import check_batch_state, expand_undirected_arcs
 
 pytestmark = pytest.mark.gpu
 
@@ -92,27 +93,22 @@ def test_fig3a_trace_rounds(rounds, Rw, Pw):
 
 # ---------------------------------------------------------------- helpers
 
-def _check_batch_state(h, o, sidx, s, eps, what):
-    P, R = h.query(sidx)
-    Po, Ro = o.query(sidx)
-    gs, gd = h.export_edges()
-    os_, od = o.export()
-    np.testing.assert_array_equal(gd, od, err_msg=f"{what}: arc dst")
-    np.testing.assert_array_equal(gs, os_, err_msg=f"{what}: arc src")
-    assert exact.terminated(R, eps), (what, np.abs(R).max())
-    ok, worst = exact.invariant_ok(h.n, gs, gd, s, h.alpha, P, R)
-    assert ok, (what, worst)
-    assert np.max(np.abs(P - Po)) <= 2 * eps, (what, np.max(np.abs(P - Po)))
-    return P, Po
+_check_batch_state = check_batch_state
 
 
-def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, relabel=-1, **over):
+def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, relabel=-1, options=None,
+                layout=ppr.LAYOUT_ARRAYS, **over):
+    """Streams `slides` batches through a handle and the oracle, checking the
+    per-batch gates.  `options`: {ppr.OPT_*: value} set through ppr_set_option
+    after create (schedule / kernel selection for the batches)."""
     st, cfg = W.make_stream(name, **over)
     eps = eps or cfg["eps"]
     g0s, g0d = st.window()
     srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], sources)
     h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=eps, mode=mode,
-                undirected=False, relabel=relabel)
+                undirected=False, relabel=relabel, layout=layout)
+    for k, v in (options or {}).items():
+        h.set_option(k, v)
     o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, eps)
     o.push(oracle.SEQ)
     for i, s in enumerate(srcs):
@@ -136,35 +132,31 @@ def test_tiny_config_all_modes_track_oracle(mode):
     _run_stream("tiny", mode, slides=12)
 
 
-@pytest.mark.parametrize("hyb,hyb_all", [("0", "0"), ("16384", "0"), ("16384", "1"), ("64", "0")])
-def test_opt_schedules_track_oracle(monkeypatch, hyb, hyb_all):
+@pytest.mark.parametrize("tail,ring_all", [(0, 0), (16384, 0), (16384, 1), (64, 0)])
+def test_opt_schedules_track_oracle(tail, ring_all):
     # Opt rounds only / rounds with the ring tail / ring from the seeds (DESIGN.md
-    # "Hybrid tail"): every schedule meets the same gates
-    monkeypatch.setenv("PPR_HYBRID", hyb)
-    monkeypatch.setenv("PPR_HYBRID_ALL", hyb_all)
-    _run_stream("tiny", "opt", slides=6)
-    _run_stream("tiny", "opt", slides=3, sources=3)
+    # "Hybrid tail"), selected through ppr_set_option: every schedule meets the same gates
+    opts = {ppr.OPT_RING_TAIL: tail, ppr.OPT_RING_ALL: ring_all}
+    _run_stream("tiny", "opt", slides=6, options=opts)
+    _run_stream("tiny", "opt", slides=3, sources=3, options=opts)
 
 
-@pytest.mark.parametrize("hyb,hyb_all", [("0", "0"), ("16384", "1")])
-def test_opt_three_edge_chains_track_oracle(monkeypatch, hyb, hyb_all):
+@pytest.mark.parametrize("tail,ring_all", [(0, 0), (16384, 1)])
+def test_opt_three_edge_chains_track_oracle(tail, ring_all):
     # the Opt push compiled with 3 edge chains per lane (push_u3.cu, chosen for
     # dense graphs) forced on the tiny config, rounds and ring schedules
-    monkeypatch.setenv("PPR_PUSH_U3", "1")
-    monkeypatch.setenv("PPR_HYBRID", hyb)
-    monkeypatch.setenv("PPR_HYBRID_ALL", hyb_all)
-    _run_stream("tiny", "opt", slides=6)
-    _run_stream("tiny", "opt", slides=3, sources=3)
+    opts = {ppr.OPT_EDGE_CHAINS: 3, ppr.OPT_RING_TAIL: tail, ppr.OPT_RING_ALL: ring_all}
+    _run_stream("tiny", "opt", slides=6, options=opts)
+    _run_stream("tiny", "opt", slides=3, sources=3, options=opts)
 
 
-@pytest.mark.parametrize("mode,hyb_all,relabel", [("opt", "0", -1), ("opt", "1", 1),
-                                                  ("eager", "0", -1), ("vanilla", "0", 1)])
-def test_packed_vertex_records_track_oracle(monkeypatch, mode, hyb_all, relabel):
+@pytest.mark.parametrize("mode,ring_all,relabel", [("opt", 0, -1), ("opt", 1, 1),
+                                                   ("eager", 0, -1), ("vanilla", 0, 1)])
+def test_packed_vertex_records_track_oracle(mode, ring_all, relabel):
     # single-source handles in the packed layout (one 32-byte {R, P, slab, d_out}
     # record per vertex): same gates as the arrays
-    monkeypatch.setenv("PPR_LAYOUT", "packed")
-    monkeypatch.setenv("PPR_HYBRID_ALL", hyb_all)
-    _run_stream("tiny", mode, slides=8, relabel=relabel)
+    _run_stream("tiny", mode, slides=8, relabel=relabel, layout=ppr.LAYOUT_PACKED,
+                options={ppr.OPT_RING_ALL: ring_all})
 
 
 @pytest.mark.parametrize("mode", ["opt", "scan", "vanilla"])
@@ -208,6 +200,14 @@ def test_tiny_config_multi_source_shared(sources):
     # (S = 40: lanes 8..31 of group 1 idle), several groups; every source of
     # every batch against the sequential oracle
     _run_stream("tiny", "shared", slides=5, sources=sources, check_every=1)
+
+
+@pytest.mark.parametrize("wave", [32, 64])
+def test_tiny_config_multi_source_shared_waves(wave):
+    # PPR_OPT_WAVE: one push launch per wave of source groups after the shared
+    # store/restore; 70 sources = 2 full groups + a partial one
+    _run_stream("tiny", "shared", slides=4, sources=70, check_every=1,
+                options={ppr.OPT_WAVE: wave})
 
 
 def test_tiny_config_multi_source_shared_relabelled_rebuild():
@@ -322,6 +322,26 @@ def test_tiny_against_power_iteration():
 
 # ---------------------------------------------------------------- restore (Lemma 3 vs Alg 1 x k)
 
+def _restore_term_scale(n, alpha, s, P, R, dout0, b):
+    """Per-vertex magnitude of the terms the batch restore sums (Lemma 3 closed
+    form): |r0| + (sum_j |op_j|(1-a)|P(v_j)| + |S0|(a 1[u=s] + |P(u)|
+    + a|r0|)) / (a d_k), or 1[u=s] + |P(u)|/a when d_k = 0 (reading R4).  Any
+    evaluation order of the closed form, and the k sequential Alg 1 calls of the
+    oracle, stay within a few ulps of this scale."""
+    isrc, idst, dsrc, ddst = (np.asarray(x, dtype=np.int64) for x in b)
+    u = np.concatenate([isrc, dsrc])
+    v = np.concatenate([idst, ddst])
+    op = np.concatenate([np.ones(len(isrc)), -np.ones(len(dsrc))])
+    S0 = np.bincount(u, weights=op, minlength=n)
+    A1 = np.bincount(u, weights=(1 - alpha) * np.abs(P[v]), minlength=n)
+    dk = dout0.astype(np.float64) + S0
+    one = np.zeros(n)
+    one[s] = 1.0
+    with np.errstate(divide="ignore", invalid="ignore"):
+        t = np.abs(R) + (A1 + np.abs(S0) * (alpha * one + np.abs(P) + alpha * np.abs(R))) / (alpha * dk)
+    return np.where(dk > 0, t, one + np.abs(P) / alpha)
+
+
 def test_restore_closed_form_matches_sequential_alg1():
     st, cfg = W.make_stream("tiny")
     g0s, g0d = st.window()
@@ -334,14 +354,21 @@ def test_restore_closed_form_matches_sequential_alg1():
     h.set_option(ppr.OPT_PUSH, 0)
     for t in range(3):
         b = st.next_batch()
-        h.apply_batch(*b)
+        before = [h.query(sidx) for sidx in range(2)]
+        dout0 = h.export_dout()
+        stt = h.apply_batch(*b)
+        assert stt["ms_restore"] > 0  # device-clock time of the restore kernel
         o.apply(*b, do_push=False)
+        touched = np.zeros(h.n, dtype=bool)
+        touched[np.concatenate([b[0], b[2]])] = True
         for sidx in range(2):
             P, R = h.query(sidx)
             Po, Ro = o.query(sidx)
             np.testing.assert_array_equal(P, Po)
-            scale = np.maximum(np.abs(Ro), 1.0)
-            assert np.max(np.abs(R - Ro) / scale) <= 1e-12
+            np.testing.assert_array_equal(R[~touched], Ro[~touched])  # restore touches only u
+            scale = _restore_term_scale(h.n, h.alpha, int(srcs[sidx]), *before[sidx], dout0, b)
+            err = np.abs(R - Ro)[touched] / scale[touched]
+            assert np.max(err) <= 1e-12, (sidx, np.max(err))
         np.testing.assert_array_equal(h.export_dout(), o.dout())
         # continue from identical states
         h.push()
@@ -492,10 +519,12 @@ def test_lj_full_size_against_oracle():
 
 def test_orkut_full_size_properties():
     """configs[2] shape at full size (undirected, 50% window, deletion-heavy
-    k = 10^4): termination and Eq. 2 at every vertex, arc count bookkeeping."""
+    k = 10^4): the arc multiset equals the expansion of the window's stream
+    edges (computed here, independently of the GPU), termination and Eq. 2 at
+    every vertex on those arcs."""
     st, cfg = W.make_stream("orkut")
     e0s, e0d = st.src[st.lo:st.hi].copy(), st.dst[st.lo:st.hi].copy()
-    arcs = W.expand_undirected(e0s, e0d)
+    arcs = expand_undirected_arcs(e0s, e0d)
     (s,) = W.pick_sources(cfg["n"], arcs[0], arcs[1], cfg["band"], 1)
     h = ppr.Ppr(cfg["n"], e0s, e0d, [s], alpha=0.15, eps=cfg["eps"], undirected=True)
     assert h.create_stats["num_arcs"] == len(arcs[0])
@@ -506,8 +535,13 @@ def test_orkut_full_size_properties():
         assert stats["num_arcs"] == 2 * (st.hi - st.lo)
     P, R = h.query()
     assert exact.terminated(R, cfg["eps"])
+    es, ed = expand_undirected_arcs(st.src[st.lo:st.hi], st.dst[st.lo:st.hi])
+    order = np.lexsort((es, ed))  # (dst, src) order of ppr_export_edges
+    es, ed = es[order], ed[order]
     gs, gd = h.export_edges()
-    ok, worst = exact.invariant_ok(cfg["n"], gs, gd, int(s), 0.15, P, R)
+    np.testing.assert_array_equal(gd, ed)
+    np.testing.assert_array_equal(gs, es)
+    ok, worst = exact.invariant_ok(cfg["n"], es, ed, int(s), 0.15, P, R)
     assert ok, worst
 
 

@@ -582,9 +582,8 @@ ppr_status enqueue_batch(ppr_ctx* h, const uint32_t* is, const uint32_t* id, uin
     launch_batch_keys(is, id, n_ins, ds, dd, n_del, h->undirected, h->n, b, 0, h->d_ctl, h->d_perm, st,
                       &launches);
     dbg_step("launch_batch_keys");
-    // Fork: the store chain (sort by (v,u), validate, apply/rebuild) stays on
-    // st; the restore chain (sort by (u,v), heads, restore) runs on st2.  The
-    // restore waits for validation so that an invalid batch mutates nothing.
+    // Fork: the store chain (sort by (v,u), heads, validate) stays on st; the
+    // restore chain's sort by (u,v) and heads run on st2 meanwhile.
     cudaEventRecord(h->ev_fork, st);
     cudaStreamWaitEvent(h->st2, h->ev_fork, 0);
     cudaStream_t s2 = h->st2;
@@ -601,23 +600,21 @@ ppr_status enqueue_batch(ppr_ctx* h, const uint32_t* is, const uint32_t* id, uin
     dbg_step("launch_heads");
     launch_heads(ku, b.ou[wu], N, b.rnu, b.uheads, &h->d_ctl->st.n_uheads, s2, &launches);
     dbg_step("launch_heads");
-    // a1: graph store
+    // a1: graph store -- validation (deletion claims, rebuild decision) on the store branch
     launch_store_validate(dg, kv, N, b, h->vb, h->d_ctl, h->force_rebuild ? 1 : 0, st, &launches);
     dbg_step("launch_store_validate");
-    cudaEventRecord(h->ev_valid, st);
-    launch_store_apply(dg, kv, N, b, h->d_ctl, st, &launches);
-    dbg_step("launch_store_apply");
-    StoreParams sp{h->slack, h->min_cap, h->pool_cap[h->active ^ 1u]};
-    const cudaError_t erb = launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches);
-    if (erb != cudaSuccess) return cuda_fail(h, erb, "store rebuild launch");
-    launch_seg_cleanup(kv, N, b, h->vb, h->d_ctl, st, &launches);
-    dbg_step("launch_seg_cleanup");
-    // a2: restore (after validation)
-    cudaStreamWaitEvent(s2, h->ev_valid, 0);
-    launch_restore(dg, ku, N, b, h->vb, h->d_ctl, s2, &launches);
-    dbg_step("launch_restore");
+    // join: the in-place apply (a1) and the restore (a2) need the validation
+    // (an invalid batch mutates nothing) and both sorts; one launch does both
     cudaEventRecord(h->ev_join, s2);
-    cudaStreamWaitEvent(st, h->ev_join, 0);  // join
+    cudaStreamWaitEvent(st, h->ev_join, 0);
+    launch_apply_restore(dg, kv, ku, N, b, h->vb, h->d_ctl, st, &launches);
+    dbg_step("launch_apply_restore");
+    // sort/merge rebuild if a slab overflowed (exits at once otherwise), then
+    // the reset of the v -> segment map
+    StoreParams sp{h->slack, h->min_cap, h->pool_cap[h->active ^ 1u]};
+    const cudaError_t erb = launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches,
+                                                 /*cleanup=*/true);
+    if (erb != cudaSuccess) return cuda_fail(h, erb, "store rebuild launch");
     *launches_out = launches;
     return PPR_OK;
 }

@@ -25,6 +25,24 @@ namespace ppr {
 
 // ---------------------------------------------------------------- radix sort
 
+// Lanes of the warp holding the same 8-bit digit d (valid lanes; an invalid
+// lane is its own group).  Eight ballots (PPR_RS_MATCH=1: one MATCH.ANY).
+__device__ __forceinline__ unsigned digit_peers(uint32_t d, bool valid) {
+#if defined(PPR_RS_MATCH) && PPR_RS_MATCH
+    (void)valid;
+    return __match_any_sync(0xffffffffu, d);
+#else
+    unsigned peers = __ballot_sync(0xffffffffu, valid);
+#pragma unroll
+    for (int bit = 0; bit < 8; bit++) {
+        const bool x = (d >> bit) & 1u;
+        const unsigned b = __ballot_sync(0xffffffffu, x);
+        peers &= x ? b : ~b;
+    }
+    return valid ? peers : (1u << (threadIdx.x & 31u));
+#endif
+}
+
 template <int ITEMS>
 __global__ void __launch_bounds__(RS_THREADS) k_rs_hist(const uint64_t* __restrict__ keys,
                                                         uint64_t n, int shift,
@@ -100,7 +118,7 @@ __global__ void __launch_bounds__(RS_THREADS) k_rs_scatter(
         uint64_t k = valid ? kin[i] : 0ull;
         uint32_t v = valid ? vin[i] : 0u;
         uint32_t d = valid ? (uint32_t)((k >> shift) & 255u) : 256u + lane;  // invalid: unique
-        unsigned peers = __match_any_sync(0xffffffffu, d);
+        unsigned peers = digit_peers(d, valid);
         unsigned rank = __popc(peers & ((1u << lane) - 1u));
         if (valid && rank == 0) s_wc[warp][d] = __popc(peers);
         __syncthreads();

@@ -170,10 +170,22 @@ __global__ void k_heads(const uint64_t* __restrict__ keys, const uint32_t* __res
 
 // ---------------------------------------------------------------- a1 store
 
+// One warp per v-segment of the (v, u)-sorted batch: run nets -> insertions I
+// and deletions Dn of v, then (Dn > 0) a scan of v's slab that claims one
+// matching slab entry per deleted copy.  The scan reads VQ consecutive slab
+// entries per lane per step (32 * VQ in flight per warp, so a hub's long
+// in-list costs len / 256 dependent steps, not len / 32) and stops once Dn
+// copies are claimed; the claimed positions are written in ascending order
+// (per-lane blocks + a warp scan), which k_store_apply relies on.
+constexpr int VQ = 8;
+
 template <bool PK>
-__global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, uint64_t N,
+__global__ void k_store_validate(const __grid_constant__ DevGraph g, const uint64_t* __restrict__ kv, uint64_t N,
                                  BatchBufs b, uint32_t* __restrict__ vseg, DevCtl* ctl,
                                  int force_rebuild) {
+    __shared__ long long s_delta;  // the CTA's net arc-count change (one global atomic per CTA)
+    if (threadIdx.x == 0) s_delta = 0;
+    __syncthreads();
     const unsigned lane = threadIdx.x & 31u;
     const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
     const uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->st.active_pool];
@@ -183,6 +195,7 @@ __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, ui
     for (uint64_t w = warp; w < nseg; w += nwarps) {
         const uint64_t i0 = b.vheads[w];
         const uint32_t v = (uint32_t)(kv[i0] >> 32);
+        const Slab sl = get_slab<PK>(g, v);  // issued before the segment walk (independent)
         const uint64_t i1 = warp_segment_end(kv, N, i0);
         uint32_t I = 0, Dn = 0;
         for (uint64_t j = i0 + lane; j < i1; j += 32) {
@@ -193,25 +206,30 @@ __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, ui
         }
         I = warp_sum_u32(I);
         Dn = warp_sum_u32(Dn);
-        const Slab sl = get_slab<PK>(g, v);
         uint32_t found = 0;
-        if (Dn > 0) {
-            for (uint32_t p0 = 0; p0 < sl.len && found < Dn; p0 += 32) {
-                const uint32_t p = p0 + lane;
-                bool claimed = false;
-                if (p < sl.len) {
-                    const uint32_t x = pool[sl.off + p];
-                    const uint64_t key = ((uint64_t)v << 32) | x;
-                    const uint64_t q = lower_bound_u64(kv, i0, i1, key);
-                    if (q < i1 && kv[q] == key) {
-                        const int32_t net = b.rnv[q];
-                        if (net < 0) claimed = atomicAdd(&b.claim[q], 1u) < (uint32_t)(-net);
+        for (uint32_t p0 = 0; Dn > 0 && p0 < sl.len && found < Dn; p0 += 32 * VQ) {
+            const uint32_t pb = p0 + lane * VQ;  // this lane's block of VQ positions
+            uint32_t x[VQ];
+#pragma unroll
+            for (int q = 0; q < VQ; q++) x[q] = pb + q < sl.len ? pool[sl.off + pb + q] : 0u;
+            uint32_t cl = 0;  // claimed positions of the block (bit q)
+#pragma unroll
+            for (int q = 0; q < VQ; q++) {
+                if (pb + q < sl.len) {
+                    const uint64_t key = ((uint64_t)v << 32) | x[q];
+                    const uint64_t r = lower_bound_u64(kv, i0, i1, key);
+                    if (r < i1 && kv[r] == key) {
+                        const int32_t net = b.rnv[r];
+                        if (net < 0 && atomicAdd(&b.claim[r], 1u) < (uint32_t)(-net)) cl |= 1u << q;
                     }
                 }
-                const unsigned m = __ballot_sync(0xffffffffu, claimed);
-                if (claimed) b.delpos[i0 + found + __popc(m & ((1u << lane) - 1u))] = p;
-                found += __popc(m);
             }
+            uint32_t tot;
+            uint32_t pos = i0 + found + warp_excl_scan_u32((uint32_t)__popc(cl), tot);
+#pragma unroll
+            for (int q = 0; q < VQ; q++)
+                if (cl & (1u << q)) b.delpos[pos++] = pb + q;
+            found += tot;
         }
         if (lane == 0) {
             b.seg_end[i0] = (uint32_t)i1;
@@ -220,21 +238,22 @@ __global__ void k_store_validate(DevGraph g, const uint64_t* __restrict__ kv, ui
             vseg[v] = (uint32_t)i0;
             if (found < Dn) set_err(ctl, KERR_NOENT);  // deletion of an absent arc
             if ((uint64_t)sl.len - found + I > sl.cap) ctl->st.rebuild = 1;
-            atomicAdd((unsigned long long*)&ctl->st.arc_delta,
-                      (unsigned long long)((long long)I - (long long)Dn));
+            atomicAdd((unsigned long long*)&s_delta, (unsigned long long)((long long)I - (long long)Dn));
         }
     }
+    __syncthreads();
+    if (threadIdx.x == 0 && s_delta)
+        atomicAdd((unsigned long long*)&ctl->st.arc_delta, (unsigned long long)s_delta);
 }
 
+// in-place slab edit of every v-segment (warps `warp` + k * nwarps)
 template <bool PK>
-__global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, BatchBufs b,
-                              DevCtl* ctl) {
-    if (*(volatile int*)&ctl->st.err != KERR_OK || *(volatile int*)&ctl->st.rebuild) return;
+__device__ __forceinline__ void apply_segments(const DevGraph& g, const uint64_t* __restrict__ kv,
+                                               const BatchBufs& b, DevCtl* ctl, uint64_t warp,
+                                               uint64_t nwarps) {
     const unsigned lane = threadIdx.x & 31u;
     const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
     uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->st.active_pool];
-    const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
-    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     for (uint64_t w = warp; w < nseg; w += nwarps) {
         const uint64_t i0 = b.vheads[w];
         const uint32_t v = (uint32_t)(kv[i0] >> 32);
@@ -275,6 +294,14 @@ __global__ void k_store_apply(DevGraph g, const uint64_t* __restrict__ kv, Batch
         }
         if (lane == 0) *lenp<PK>(g, v) = keep + I;
     }
+}
+
+template <bool PK>
+__global__ void k_store_apply(const __grid_constant__ DevGraph g, const uint64_t* __restrict__ kv,
+                              BatchBufs b, DevCtl* ctl) {
+    if (*(volatile int*)&ctl->st.err != KERR_OK || *(volatile int*)&ctl->st.rebuild) return;
+    apply_segments<PK>(g, kv, b, ctl, ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5,
+                       ((uint64_t)gridDim.x * blockDim.x) >> 5);
 }
 
 // ---------------------------------------------------------------- a1 rebuild
@@ -340,11 +367,9 @@ __device__ uint32_t copy_merged_warp(const uint32_t* src, uint32_t* dst, const S
 }
 
 template <bool PK>
-__global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64_t* __restrict__ kv,
-                                                        BatchBufs b, VertexBufs vb, double slack,
-                                                        uint32_t min_cap, uint64_t alt_cap,
-                                                        DevCtl* ctl) {
-    if (*(volatile int*)&ctl->st.err != KERR_OK || !*(volatile int*)&ctl->st.rebuild) return;
+__device__ __forceinline__ void rebuild_body(const DevGraph& g, const uint64_t* __restrict__ kv,
+                                             const BatchBufs& b, const VertexBufs& vb, double slack,
+                                             uint32_t min_cap, uint64_t alt_cap, DevCtl* ctl) {
     __shared__ uint32_t s_warp[RB_THREADS / 32 + 1];
     __shared__ unsigned long long s_warp64[RB_THREADS / 32 + 1];
     const unsigned act = *(volatile unsigned*)&ctl->st.active_pool;
@@ -438,6 +463,24 @@ __global__ void __launch_bounds__(RB_THREADS) k_rebuild(DevGraph g, const uint64
     if (blockIdx.x == 0 && threadIdx.x == 0) ctl->st.active_pool = act ^ 1u;
 }
 
+// The rebuild (only if a slab would overflow; the decision is uniform: it was
+// made by the validation before this launch) and, with `cleanup`, the reset
+// of the batch's v -> segment map (k_seg_cleanup folded in: one launch fewer)
+template <bool PK>
+__global__ void __launch_bounds__(RB_THREADS) k_rebuild(const __grid_constant__ DevGraph g,
+                                                        const uint64_t* __restrict__ kv, BatchBufs b,
+                                                        VertexBufs vb, double slack, uint32_t min_cap,
+                                                        uint64_t alt_cap, DevCtl* ctl, int cleanup) {
+    if (*(volatile int*)&ctl->st.err == KERR_OK && *(volatile int*)&ctl->st.rebuild)
+        rebuild_body<PK>(g, kv, b, vb, slack, min_cap, alt_cap, ctl);
+    if (cleanup) {
+        const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
+        for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nseg;
+             w += (uint64_t)gridDim.x * blockDim.x)
+            vb.vseg[kv[b.vheads[w]] >> 32] = NONE;
+    }
+}
+
 __global__ void k_seg_cleanup(const uint64_t* __restrict__ kv, BatchBufs b,
                               uint32_t* __restrict__ vseg, DevCtl* ctl) {
     const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
@@ -448,51 +491,116 @@ __global__ void k_seg_cleanup(const uint64_t* __restrict__ kv, BatchBufs b,
 
 // ---------------------------------------------------------------- a2 restore
 
+// Lemma 3 closed form for the u-segment starting at i0 and the sources
+// si = s0, s0 + ds, ... (one thread per segment: s0 = 0, ds = 1; one warp per
+// segment: s0 = lane, ds = 32 -- the S residuals of u are one vertex-major row,
+// so the lanes' loads coalesce).  Returns false if the segment's updates all
+// cancelled (nothing to restore).
 template <bool PK>
-__global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t N, BatchBufs b,
-                          uint32_t* __restrict__ touched, DevCtl* ctl) {
+__device__ __forceinline__ bool restore_segment(const DevGraph& g, const uint64_t* __restrict__ ku,
+                                                uint64_t N, const BatchBufs& b, uint64_t i0,
+                                                uint32_t s0, uint32_t ds, bool write_dout) {
+    const double a = g.alpha;
+    const uint32_t u = (uint32_t)(ku[i0] >> 32);
+    int64_t S0 = 0;
+    bool any = false;
+    uint64_t i1 = i0;
+    for (; i1 < N && (ku[i1] >> 32) == u; i1++) {
+        if (is_run_head(ku, i1, i0)) {
+            const int32_t net = b.rnu[i1];
+            S0 += net;
+            any |= net != 0;
+        }
+    }
+    if (!any) return false;
+    const int64_t dk = (int64_t)*doutp<PK>(g, u) + S0;  // post-batch d_out(u) (reading R3)
+    for (uint32_t si = s0; si < g.S; si += ds) {
+        double s1 = 0.0;
+        for (uint64_t j = i0; j < i1; j++) {
+            if (!is_run_head(ku, j, i0)) continue;
+            const int32_t net = b.rnu[j];
+            if (net != 0) s1 += (double)net * *Pp<PK>(g, si, (uint32_t)ku[j]);
+        }
+        const double S1 = (1.0 - a) * s1;
+        const double one = (u == g.sources[si]) ? 1.0 : 0.0;
+        const double pu = *Pp<PK>(g, si, u);
+        const double r0 = *Rp<PK>(g, si, u);
+        double r;
+        if (dk > 0)
+            r = r0 + (S1 + (double)S0 * (a * one - pu - a * r0)) / (a * (double)dk);
+        else
+            r = one - pu / a;  // Eq. 2 with an empty sum (reading R4)
+        *Rp<PK>(g, si, u) = r;
+    }
+    if (ds == 32) __syncwarp();  // every lane has read d_out(u) above
+    if (write_dout) *doutp<PK>(g, u) = (uint32_t)dk;
+    return true;
+}
+
+// every u-segment: thread per segment (S == 1) or warp per segment (S > 1);
+// `item` / `nitems` index threads or warps of the participating blocks
+template <bool PK>
+__device__ __forceinline__ void restore_segments(const DevGraph& g, const uint64_t* __restrict__ ku,
+                                                 uint64_t N, const BatchBufs& b,
+                                                 uint32_t* __restrict__ touched, DevCtl* ctl,
+                                                 uint64_t item, uint64_t nitems) {
+    const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_uheads;
+    const unsigned lane = threadIdx.x & 31u;
+    if (g.S == 1) {
+        for (uint64_t k = item; k < nseg; k += nitems) {
+            const uint64_t i0 = b.uheads[k];
+            if (restore_segment<PK>(g, ku, N, b, i0, 0, 1, true))
+                touched[atomicAdd(&ctl->st.n_touched, 1u)] = (uint32_t)(ku[i0] >> 32);
+        }
+    } else {
+        for (uint64_t k = item; k < nseg; k += nitems) {
+            const uint64_t i0 = b.uheads[k];
+            if (restore_segment<PK>(g, ku, N, b, i0, lane, 32, lane == 0) && lane == 0)
+                touched[atomicAdd(&ctl->st.n_touched, 1u)] = (uint32_t)(ku[i0] >> 32);
+        }
+    }
+}
+
+// restore grid: threads (S == 1) or warps (S > 1) over the u-segments
+inline unsigned restore_blocks(uint64_t N, uint32_t S, unsigned threads) {
+    const uint64_t items = S == 1 ? N : N * 32;
+    uint64_t blocks = (items + threads - 1) / threads;
+    if (blocks < 1) blocks = 1;
+    if (blocks > 148 * 32) blocks = 148 * 32;
+    return (unsigned)blocks;
+}
+
+template <bool PK>
+__global__ void k_restore(const __grid_constant__ DevGraph g, const uint64_t* __restrict__ ku,
+                          uint64_t N, BatchBufs b, uint32_t* __restrict__ touched, DevCtl* ctl) {
     if (*(volatile int*)&ctl->st.err != KERR_OK) return;
     if (threadIdx.x == 0) atomicMin(&ctl->st.t_restore[0], globaltimer_ns());
-    const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_uheads;
-    const double a = g.alpha;
-    for (uint64_t k = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; k < nseg;
-         k += (uint64_t)gridDim.x * blockDim.x) {
-        const uint64_t i0 = b.uheads[k];
-        const uint32_t u = (uint32_t)(ku[i0] >> 32);
-        int64_t S0 = 0;
-        bool any = false;
-        uint64_t i1 = i0;
-        for (; i1 < N && (ku[i1] >> 32) == u; i1++) {
-            if (is_run_head(ku, i1, i0)) {
-                const int32_t net = b.rnu[i1];
-                S0 += net;
-                any |= net != 0;
-            }
-        }
-        if (!any) continue;
-        const int64_t dk = (int64_t)*doutp<PK>(g, u) + S0;  // post-batch d_out(u) (reading R3)
-        *doutp<PK>(g, u) = (uint32_t)dk;
-        for (uint32_t si = 0; si < g.S; si++) {
-            double s1 = 0.0;
-            for (uint64_t j = i0; j < i1; j++) {
-                if (!is_run_head(ku, j, i0)) continue;
-                const int32_t net = b.rnu[j];
-                if (net != 0) s1 += (double)net * *Pp<PK>(g, si, (uint32_t)ku[j]);
-            }
-            const double S1 = (1.0 - a) * s1;
-            const double one = (u == g.sources[si]) ? 1.0 : 0.0;
-            const double pu = *Pp<PK>(g, si, u);
-            const double r0 = *Rp<PK>(g, si, u);
-            double r;
-            if (dk > 0)
-                r = r0 + (S1 + (double)S0 * (a * one - pu - a * r0)) / (a * (double)dk);
-            else
-                r = one - pu / a;  // Eq. 2 with an empty sum (reading R4)
-            *Rp<PK>(g, si, u) = r;
-        }
-        const unsigned pos = atomicAdd(&ctl->st.n_touched, 1u);
-        touched[pos] = u;
+    const uint64_t tid = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    const uint64_t nth = (uint64_t)gridDim.x * blockDim.x;
+    if (g.S == 1) restore_segments<PK>(g, ku, N, b, touched, ctl, tid, nth);
+    else restore_segments<PK>(g, ku, N, b, touched, ctl, tid >> 5, nth >> 5);
+    __syncthreads();
+    if (threadIdx.x == 0) atomicMax(&ctl->st.t_restore[1], globaltimer_ns());
+}
+
+// small-batch path: the in-place apply (blocks [0, apply_blocks)) and the
+// restore (the other blocks) in one launch -- both need only the validation
+template <bool PK>
+__global__ void k_apply_restore(const __grid_constant__ DevGraph g, const uint64_t* __restrict__ kv,
+                                const uint64_t* __restrict__ ku, uint64_t N, BatchBufs b,
+                                uint32_t* __restrict__ touched, DevCtl* ctl, unsigned apply_blocks) {
+    if (*(volatile int*)&ctl->st.err != KERR_OK) return;
+    if (blockIdx.x < apply_blocks) {
+        if (!*(volatile int*)&ctl->st.rebuild)
+            apply_segments<PK>(g, kv, b, ctl, ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5,
+                               ((uint64_t)apply_blocks * blockDim.x) >> 5);
+        return;
     }
+    if (threadIdx.x == 0) atomicMin(&ctl->st.t_restore[0], globaltimer_ns());
+    const uint64_t tid = (uint64_t)(blockIdx.x - apply_blocks) * blockDim.x + threadIdx.x;
+    const uint64_t nth = (uint64_t)(gridDim.x - apply_blocks) * blockDim.x;
+    if (g.S == 1) restore_segments<PK>(g, ku, N, b, touched, ctl, tid, nth);
+    else restore_segments<PK>(g, ku, N, b, touched, ctl, tid >> 5, nth >> 5);
     __syncthreads();
     if (threadIdx.x == 0) atomicMax(&ctl->st.t_restore[1], globaltimer_ns());
 }
@@ -501,7 +609,7 @@ __global__ void k_restore(DevGraph g, const uint64_t* __restrict__ ku, uint64_t 
 
 template <bool PK>
 __global__ void k_build_count(const uint32_t* __restrict__ src, const uint32_t* __restrict__ dst,
-                              uint64_t m, int undirected, DevGraph g) {
+                              uint64_t m, int undirected, const __grid_constant__ DevGraph g) {
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
          i += (uint64_t)gridDim.x * blockDim.x) {
         const uint32_t u = src[i], v = dst[i];
@@ -515,7 +623,7 @@ __global__ void k_build_count(const uint32_t* __restrict__ src, const uint32_t* 
 }
 
 template <bool PK>
-__global__ void k_caps_from_len(DevGraph g, uint32_t* __restrict__ newcap, double slack,
+__global__ void k_caps_from_len(const __grid_constant__ DevGraph g, uint32_t* __restrict__ newcap, double slack,
                                 uint32_t min_cap) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x) {
@@ -526,7 +634,7 @@ __global__ void k_caps_from_len(DevGraph g, uint32_t* __restrict__ newcap, doubl
 }
 
 template <bool PK>
-__global__ void k_set_slabs(DevGraph g, const unsigned long long* __restrict__ off,
+__global__ void k_set_slabs(const __grid_constant__ DevGraph g, const unsigned long long* __restrict__ off,
                             const uint32_t* __restrict__ cap) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x) {
@@ -540,7 +648,7 @@ __global__ void k_set_slabs(DevGraph g, const unsigned long long* __restrict__ o
 
 template <bool PK>
 __global__ void k_build_fill(const uint32_t* __restrict__ src, const uint32_t* __restrict__ dst,
-                             uint64_t m, int undirected, DevGraph g) {
+                             uint64_t m, int undirected, const __grid_constant__ DevGraph g) {
     uint32_t* pool = g.pool[0];
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
          i += (uint64_t)gridDim.x * blockDim.x) {
@@ -555,21 +663,21 @@ __global__ void k_build_fill(const uint32_t* __restrict__ src, const uint32_t* _
 }
 
 template <bool PK>
-__global__ void k_init_state(DevGraph g) {
+__global__ void k_init_state(const __grid_constant__ DevGraph g) {
     // P = 0 and R = 0 are set by memset; R(s) = 1 for each source (Fig. 3 a(1))
     for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < g.S; i += gridDim.x * blockDim.x)
         *Rp<PK>(g, i, g.sources[i]) = 1.0;
 }
 
 template <bool PK>
-__global__ void k_len_to_u32(DevGraph g, uint32_t* __restrict__ out) {
+__global__ void k_len_to_u32(const __grid_constant__ DevGraph g, uint32_t* __restrict__ out) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x)
         out[v] = *lenp<PK>(g, (uint32_t)v);
 }
 
 template <bool PK>
-__global__ void k_export(DevGraph g, int active, const unsigned long long* __restrict__ off,
+__global__ void k_export(const __grid_constant__ DevGraph g, int active, const unsigned long long* __restrict__ off,
                          uint64_t* __restrict__ keys, const uint32_t* __restrict__ inv) {
     const uint32_t* pool = g.pool[active];
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
@@ -645,7 +753,7 @@ __global__ void k_gather_u32(const uint32_t* __restrict__ src, const uint32_t* _
 }
 
 // packed layout: P, R, d_out out of the records (query / export / reset)
-__global__ void k_gather_rec(DevGraph g, double* __restrict__ P, double* __restrict__ R,
+__global__ void k_gather_rec(const __grid_constant__ DevGraph g, double* __restrict__ P, double* __restrict__ R,
                              uint32_t* __restrict__ dout, int zero_pr,
                              const uint32_t* __restrict__ perm) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
@@ -715,7 +823,7 @@ void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const
 
 cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                                  const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
-                                 cudaStream_t st, uint32_t* launches) {
+                                 cudaStream_t st, uint32_t* launches, bool cleanup) {
     (void)N;
     const void* fn = g.rec ? (const void*)k_rebuild<true> : (const void*)k_rebuild<false>;
     int per_sm = 0, sms = 0, dev = 0;
@@ -732,7 +840,8 @@ cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t
     uint32_t min_cap = sp.min_cap;
     uint64_t alt_cap = sp.alt_cap;
     DevCtl* c = ctl;
-    void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &alt_cap, &c};
+    int cl = cleanup ? 1 : 0;
+    void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &alt_cap, &c, &cl};
     e = cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(RB_THREADS), args, 0, st);
     ++*launches;
     return e;
@@ -746,7 +855,16 @@ void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, cons
 
 void launch_restore(const DevGraph& g, const uint64_t* ku, uint64_t N, const BatchBufs& b,
                     const VertexBufs& vb, DevCtl* ctl, cudaStream_t st, uint32_t* launches) {
-    LAUNCH_PK(k_restore)<<<grid_for(N, 128), 128, 0, st>>>(g, ku, N, b, vb.touched, ctl);
+    LAUNCH_PK(k_restore)<<<restore_blocks(N, g.S, 128), 128, 0, st>>>(g, ku, N, b, vb.touched, ctl);
+    ++*launches;
+}
+
+void launch_apply_restore(const DevGraph& g, const uint64_t* kv, const uint64_t* ku, uint64_t N,
+                          const BatchBufs& b, const VertexBufs& vb, DevCtl* ctl, cudaStream_t st,
+                          uint32_t* launches) {
+    const unsigned ab = grid_for(N * 32, 256);
+    LAUNCH_PK(k_apply_restore)<<<ab + restore_blocks(N, g.S, 256), 256, 0, st>>>(g, kv, ku, N, b,
+                                                                              vb.touched, ctl, ab);
     ++*launches;
 }
 

@@ -65,12 +65,17 @@ void launch_store_validate(const DevGraph& g, const uint64_t* kv, uint64_t N, co
 void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                         DevCtl* ctl, cudaStream_t st, uint32_t* launches);
 // a1: sort/merge rebuild into the other pool (skipped unless DevCtl::rebuild)
+// (cleanup: also reset the v -> segment map, i.e. launch_seg_cleanup folded in)
 cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                                  const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
-                                 cudaStream_t st, uint32_t* launches);
+                                 cudaStream_t st, uint32_t* launches, bool cleanup = false);
 void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, const VertexBufs& vb,
                         DevCtl* ctl, cudaStream_t st, uint32_t* launches);
 
+// small-batch path: a1 in-place apply and a2 restore in one launch (after validation)
+void launch_apply_restore(const DevGraph& g, const uint64_t* kv, const uint64_t* ku, uint64_t N,
+                          const BatchBufs& b, const VertexBufs& vb, DevCtl* ctl, cudaStream_t st,
+                          uint32_t* launches);
 // a2: Lemma 3 closed-form restore per touched u (and d_out update)
 void launch_restore(const DevGraph& g, const uint64_t* ku, uint64_t N, const BatchBufs& b,
                     const VertexBufs& vb, DevCtl* ctl, cudaStream_t st, uint32_t* launches);

@@ -159,6 +159,27 @@ def test_packed_vertex_records_track_oracle(mode, ring_all, relabel):
                 options={ppr.OPT_RING_ALL: ring_all})
 
 
+@pytest.mark.parametrize("n_arcs", [2 ** 18, 2 ** 18 + 1])
+def test_radix_sort_tile_switch(n_arcs):
+    # batches at the radix sort's 2^18-key tile switch and one key past it
+    # (512-key tiles + fused scan vs 4096-key tiles + scan kernel), with
+    # duplicates and an insert/delete pair of the same arc
+    n = 200_000
+    src, dst = W.rmat_stream(n, 1_000_000, seed=9, abc=W.SHAPED)
+    w0 = 500_000
+    (s,) = W.pick_sources(n, src[:w0], dst[:w0], 1000, 1)
+    h = ppr.Ppr(n, src[:w0], dst[:w0], [s], alpha=0.15, eps=1e-8)
+    o = oracle.Oracle(n, src[:w0], dst[:w0], [s], 0.15, 1e-8)
+    o.push(oracle.SEQ)
+    ni = n_arcs // 2
+    nd = n_arcs - ni
+    ins = (np.concatenate([src[w0:w0 + ni - 3], src[:2], [7]]), np.concatenate([dst[w0:w0 + ni - 3], dst[:2], [8]]))
+    dels = (np.concatenate([src[:nd - 1], [7]]), np.concatenate([dst[:nd - 1], [8]]))
+    h.apply_batch(*ins, *dels)
+    o.apply(*ins, *dels)
+    _check_batch_state(h, o, 0, int(s), 1e-8, f"batch of {n_arcs} arcs")
+
+
 @pytest.mark.parametrize("mode", ["opt", "scan", "vanilla"])
 def test_tiny_config_degree_relabelled(mode):
     # internal degree-ordered ids: every id at the boundary must stay external
@@ -323,11 +344,12 @@ def test_tiny_against_power_iteration():
 # ---------------------------------------------------------------- restore (Lemma 3 vs Alg 1 x k)
 
 def _restore_term_scale(n, alpha, s, P, R, dout0, b):
-    """Per-vertex magnitude of the terms the batch restore sums (Lemma 3 closed
-    form): |r0| + (sum_j |op_j|(1-a)|P(v_j)| + |S0|(a 1[u=s] + |P(u)|
-    + a|r0|)) / (a d_k), or 1[u=s] + |P(u)|/a when d_k = 0 (reading R4).  Any
-    evaluation order of the closed form, and the k sequential Alg 1 calls of the
-    oracle, stay within a few ulps of this scale."""
+    """Per-vertex magnitude of the terms either evaluation sums: the batch
+    closed form (Lemma 3 proof: |r0| + (sum_j |op_j|(1-a)|P(v_j)| +
+    |S0|(a 1[u=s] + |P(u)| + a|r0|)) / (a d_k), or 1[u=s] + |P(u)|/a when d_k = 0,
+    reading R4) and the oracle's k sequential Alg 1 calls (the
+    largest intermediate |R(u)| and update term, with the intermediate
+    degrees).  Both evaluations are exact up to a few ulps of this scale."""
     isrc, idst, dsrc, ddst = (np.asarray(x, dtype=np.int64) for x in b)
     u = np.concatenate([isrc, dsrc])
     v = np.concatenate([idst, ddst])
@@ -339,7 +361,20 @@ def _restore_term_scale(n, alpha, s, P, R, dout0, b):
     one[s] = 1.0
     with np.errstate(divide="ignore", invalid="ignore"):
         t = np.abs(R) + (A1 + np.abs(S0) * (alpha * one + np.abs(P) + alpha * np.abs(R))) / (alpha * dk)
-    return np.where(dk > 0, t, one + np.abs(P) / alpha)
+    scale = np.where(dk > 0, t, one + np.abs(P) / alpha)
+    # the sequential path: insertions then deletions, in order (oracle CPU-Seq)
+    d = dout0.astype(np.int64).copy()
+    r = np.array(R, dtype=np.float64)
+    for uu, vv, o in zip(u.tolist(), v.tolist(), op.tolist()):
+        d[uu] += int(o)
+        if d[uu] > 0:
+            term = ((1 - alpha) * abs(P[vv]) + abs(P[uu]) + alpha * abs(r[uu]) + alpha * one[uu]) / (alpha * d[uu])
+            r[uu] += o * ((1 - alpha) * P[vv] - P[uu] - alpha * r[uu] + alpha * one[uu]) / (alpha * d[uu])
+        else:
+            term = one[uu] + abs(P[uu]) / alpha
+            r[uu] = one[uu] - P[uu] / alpha
+        scale[uu] = max(scale[uu], term, abs(r[uu]))
+    return scale
 
 
 def test_restore_closed_form_matches_sequential_alg1():
@@ -367,7 +402,9 @@ def test_restore_closed_form_matches_sequential_alg1():
             np.testing.assert_array_equal(P, Po)
             np.testing.assert_array_equal(R[~touched], Ro[~touched])  # restore touches only u
             scale = _restore_term_scale(h.n, h.alpha, int(srcs[sidx]), *before[sidx], dout0, b)
-            err = np.abs(R - Ro)[touched] / scale[touched]
+            d, sc = np.abs(R - Ro)[touched], scale[touched]
+            assert np.all(d[sc == 0] == 0)  # all terms zero: both sides exactly 0
+            err = d[sc > 0] / sc[sc > 0]
             assert np.max(err) <= 1e-12, (sidx, np.max(err))
         np.testing.assert_array_equal(h.export_dout(), o.dout())
         # continue from identical states

@@ -47,8 +47,12 @@ template <int ITEMS>
 __global__ void __launch_bounds__(RS_THREADS) k_rs_hist(const uint64_t* __restrict__ keys,
                                                         uint64_t n, int shift,
                                                         uint32_t* __restrict__ hist,
-                                                        uint32_t ntiles) {
+                                                        uint32_t ntiles,
+                                                        uint32_t* __restrict__ hist_zero = nullptr) {
     __shared__ uint32_t s_h[256];
+    if (hist_zero)
+        for (uint32_t i = blockIdx.x * RS_THREADS + threadIdx.x; i < 256u * ntiles; i += gridDim.x * RS_THREADS)
+            hist_zero[i] = 0u;
     s_h[threadIdx.x] = 0;
     __syncthreads();
     const uint64_t base = (uint64_t)blockIdx.x * RS_THREADS * ITEMS;
@@ -81,11 +85,17 @@ __global__ void __launch_bounds__(RS_THREADS) k_rs_scan(uint32_t* __restrict__ h
 
 // FUSED: the tile offsets are summed here from the raw per-tile counts
 // (ntiles <= RS_FUSED_MAX_TILES), otherwise k_rs_scan has prepared them.
-template <int ITEMS, bool FUSED>
+// CHAIN (small sorts, FUSED): the scatter also builds the NEXT pass's per-tile
+// histogram -- each key it writes to position pos adds 1 to (next digit, pos's
+// tile) of hist_next -- and zeroes hist_zero (the buffer the pass after next will
+// fill), so only the first pass needs a histogram kernel.  Three buffers rotate:
+// pass p reads H[p % 3], fills H[(p + 1) % 3], zeroes H[(p + 2) % 3].
+template <int ITEMS, bool FUSED, bool CHAIN = false>
 __global__ void __launch_bounds__(RS_THREADS) k_rs_scatter(
     const uint64_t* __restrict__ kin, const uint32_t* __restrict__ vin,
     uint64_t* __restrict__ kout, uint32_t* __restrict__ vout, uint64_t n, int shift,
-    const uint32_t* __restrict__ hist, uint32_t ntiles) {
+    const uint32_t* __restrict__ hist, uint32_t ntiles, int next_shift = -1,
+    uint32_t* __restrict__ hist_next = nullptr, uint32_t* __restrict__ hist_zero = nullptr) {
     constexpr int NW = RS_THREADS / 32;
     __shared__ uint32_t s_warp[NW + 1];
     __shared__ uint32_t s_run[256];      // next output position per digit
@@ -138,8 +148,14 @@ __global__ void __launch_bounds__(RS_THREADS) k_rs_scatter(
             uint32_t pos = s_wo[warp][d] + rank;
             kout[pos] = k;
             vout[pos] = v;
+            if (CHAIN && next_shift >= 0)
+                atomicAdd(&hist_next[(uint64_t)((k >> next_shift) & 255u) * ntiles +
+                                     pos / (RS_THREADS * ITEMS)], 1u);
         }
     }
+    if (CHAIN && hist_zero)
+        for (uint32_t i = blockIdx.x * RS_THREADS + t; i < 256u * ntiles; i += gridDim.x * RS_THREADS)
+            hist_zero[i] = 0u;
 }
 
 int radix_sort_pairs(uint64_t* k0, uint32_t* v0, uint64_t* k1, uint32_t* v1, uint64_t n,
@@ -152,6 +168,27 @@ int radix_sort_pairs(uint64_t* k0, uint32_t* v0, uint64_t* k1, uint32_t* v1, uin
     uint64_t *ki = k0, *ko = k1;
     uint32_t *vi = v0, *vo = v1;
     int where = 0;
+    if (small && fused) {  // chained passes: one histogram kernel, then one scatter per pass
+        const uint64_t stride = 256ull * (ntiles + 1);
+        uint32_t* H[3] = {hist, hist + stride, hist + 2 * stride};
+        k_rs_hist<2><<<ntiles, RS_THREADS, 0, st>>>(ki, n, shifts[0], H[0], ntiles, H[1]);
+        ++*launches;
+        for (int p = 0; p < npasses; p++) {
+            const bool last = p + 1 == npasses;
+            k_rs_scatter<2, true, true><<<ntiles, RS_THREADS, 0, st>>>(
+                ki, vi, ko, vo, n, shifts[p], H[p % 3], ntiles, last ? -1 : shifts[p + 1],
+                H[(p + 1) % 3], last ? nullptr : H[(p + 2) % 3]);
+            ++*launches;
+            uint64_t* tk = ki;
+            ki = ko;
+            ko = tk;
+            uint32_t* tv = vi;
+            vi = vo;
+            vo = tv;
+            where ^= 1;
+        }
+        return where;
+    }
     for (int p = 0; p < npasses; p++) {
         if (small) {
             k_rs_hist<2><<<ntiles, RS_THREADS, 0, st>>>(ki, n, shifts[p], hist, ntiles);

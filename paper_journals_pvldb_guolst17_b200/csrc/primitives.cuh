@@ -11,16 +11,20 @@ constexpr int RS_THREADS = 256;
 // keys per thread per pass: small batches use short tiles so that many CTAs
 // share a pass, large ones long tiles so that the per-tile histograms stay few
 inline int rs_items(uint64_t n) { return n <= (1u << 18) ? 2 : 16; }
+constexpr uint32_t RS_FUSED_MAX_TILES = 64;  // at most this many tiles: no separate scan kernel
 inline uint64_t rs_tiles(uint64_t n) {
     const uint64_t tile = (uint64_t)RS_THREADS * rs_items(n);
     return (n + tile - 1) / tile;
 }
-constexpr uint32_t RS_FUSED_MAX_TILES = 64;  // at most this many tiles: no separate scan kernel
 // scratch entries (u32) the sort needs for n keys
 // (valid for every sort of m <= n keys)
 inline uint64_t rs_hist_entries(uint64_t n) {
     uint64_t t = rs_tiles(n), ts = rs_tiles(n < (1u << 18) ? n : (1u << 18));
-    return 256 * ((t > ts ? t : ts) + 1) + 256;
+    const uint64_t one = 256 * ((t > ts ? t : ts) + 1) + 256;
+    // chained small sorts (<= RS_FUSED_MAX_TILES tiles) rotate three histograms
+    const uint64_t tc = t < RS_FUSED_MAX_TILES ? t : RS_FUSED_MAX_TILES;
+    const uint64_t three = 3 * 256 * (tc + 1);
+    return one > three ? one : three;
 }
 
 // Sorts n pairs by the bits [shift, shift+8) for every shift in `shifts`

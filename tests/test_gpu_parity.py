@@ -159,10 +159,11 @@ def test_packed_vertex_records_track_oracle(mode, ring_all, relabel):
                 options={ppr.OPT_RING_ALL: ring_all})
 
 
-@pytest.mark.parametrize("n_arcs", [2 ** 18, 2 ** 18 + 1])
+@pytest.mark.parametrize("n_arcs", [32768, 32769, 2 ** 18, 2 ** 18 + 1])
 def test_radix_sort_tile_switch(n_arcs):
-    # batches at the radix sort's 2^18-key tile switch and one key past it
-    # (512-key tiles + fused scan vs 4096-key tiles + scan kernel), with
+    # batches at the radix sort's switches and one key past each: <= 64 tiles of
+    # 512 keys (chained passes: the scatter builds the next pass's histogram),
+    # more tiles with a scan kernel, and past 2^18 keys 4096-key tiles; with
     # duplicates and an insert/delete pair of the same arc
     n = 200_000
     src, dst = W.rmat_stream(n, 1_000_000, seed=9, abc=W.SHAPED)

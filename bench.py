@@ -50,11 +50,14 @@ ROOT = os.path.dirname(os.path.abspath(__file__))
 sys.path.insert(0, ROOT)
 
 # algorithmic bytes per unit: a pushed edge is 24 B =
-# 8 B of walk (v id + d_out(v)) + 16 B of R(v) read+write; a pushed vertex 52 B.
-# The shared multi-source kernel walks an in-arc once per (source group, arc),
-# so its bytes are 8 per walked arc + 16 per (source, arc) propagation.
-B_EDGE, B_VERTEX, B_ARC = 24, 52, 56
-B_WALK, B_PROP = 8, 16
+# 8 B of walk (v id + d_out(v)) + 16 B of R(v) read+write; a pushed vertex 52 B =
+# 32 B of R(u), P(u) read+write per (source, vertex) + 20 B of frontier id, slab
+# off/len and next-frontier write per frontier entry.  The shared multi-source
+# kernel walks an in-arc once per (source group, arc) and reads one slab / writes
+# one frontier id per (vertex, group) entry, so its bytes are 8 per walked arc +
+# 16 per (source, arc) propagation + 32 per (source, vertex) push + 20 per entry;
+# for one source per entry this is exactly 24 per edge + 52 per vertex.
+B_WALK, B_PROP, B_PUSH, B_ENTRY = 8, 16, 32, 20
 
 
 def parse():
@@ -559,7 +562,8 @@ def measure(args, cx, workload, S_total, with_e2e, with_cpu):
     e_r0 = sum(s["pushed_edges"] for s in stats) / steps
     v_r0 = sum(s["pushes"] for s in stats) / steps
     w_r0 = sum(s["walk_edges"] for s in stats) / steps
-    bytes_step = (B_WALK * w_r0 + B_PROP * e_r0 + B_VERTEX * v_r0)
+    n_r0 = sum(s["entries"] for s in stats) / steps
+    bytes_step = B_WALK * w_r0 + B_PROP * e_r0 + B_PUSH * v_r0 + B_ENTRY * n_r0
     push_step = sum(push_ms) / steps
     achieved = bytes_step / (push_step / 1e3) / 1e9 if push_step > 0 else 0.0
     tr = profile_traffic(workload) if len(my_srcs) == 1 else None
@@ -598,6 +602,7 @@ def measure(args, cx, workload, S_total, with_e2e, with_cpu):
             "ms_push_neg": sum(s["ms_push_neg"] for s in stats) / steps,
             "pushed_edges_per_s": tot["pushed_edges"] / (T / 1e3),
             "pushes_per_step": tot["pushes"] / steps,
+            "walk_edges_per_step_rank0": w_r0, "entries_per_step_rank0": n_r0,
             "pushed_edges_per_step": tot["pushed_edges"] / steps,
             "iters_per_step": sum(s["iters_pos"] + s["iters_neg"] for s in stats) / steps,
             "rebuilds": sum(s["rebuilt"] for s in stats),

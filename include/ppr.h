@@ -151,6 +151,9 @@ typedef struct {
     float ms_push_pos, ms_push_neg; /* device clock inside the push launch: seed + rounds of the
                                        POS phase (a3-a4) and of the NEG phase (a5); 0 for
                                        PPR_MODE_SORTAGG (host-driven rounds) */
+    uint64_t entries;               /* frontier entries processed: PPR_MODE_SHARED counts (vertex,
+                                       32-source group) rows with a pushing lane; other modes:
+                                       = pushes */
 } ppr_batch_stats;
 
 /* Creates a handle: builds the slab store for g, sets P_s = 0 and R_s = e_s

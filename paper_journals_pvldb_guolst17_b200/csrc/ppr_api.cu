@@ -46,12 +46,11 @@ struct GraphKey {
     uint64_t epoch = 0, cap0 = 0, cap1 = 0;
     const void* pool0 = nullptr;
     const void* pool1 = nullptr;
-    unsigned active = 0;  // the rebuild's capacity check (StoreParams::alt_cap) is baked in per active pool
     bool operator==(const GraphKey& o) const {
         return n_ins == o.n_ins && n_del == o.n_del && push == o.push && mode == o.mode &&
                max_iters == o.max_iters && timing == o.timing && force_rebuild == o.force_rebuild &&
                epoch == o.epoch && cap0 == o.cap0 && cap1 == o.cap1 && pool0 == o.pool0 &&
-               pool1 == o.pool1 && active == o.active;
+               pool1 == o.pool1;
     }
 };
 
@@ -326,6 +325,7 @@ void fill_stats(ppr_ctx* h, ppr_batch_stats* s, uint32_t launches, bool timed,
     s->pushes = c.pushes;
     s->pushed_edges = c.pushed_edges;
     s->walk_edges = h->mode == PPR_MODE_SHARED ? c.walk_edges : c.pushed_edges;
+    s->entries = h->mode == PPR_MODE_SHARED ? c.entries : c.pushes;
     s->max_frontier = c.max_frontier;
     s->touched = (uint64_t)c.n_touched * h->S;
     s->num_arcs = h->m;
@@ -611,7 +611,7 @@ ppr_status enqueue_batch(ppr_ctx* h, const uint32_t* is, const uint32_t* id, uin
     dbg_step("launch_apply_restore");
     // sort/merge rebuild if a slab overflowed (exits at once otherwise), then
     // the reset of the v -> segment map
-    StoreParams sp{h->slack, h->min_cap, h->pool_cap[h->active ^ 1u]};
+    StoreParams sp{h->slack, h->min_cap, h->pool_cap[0], h->pool_cap[1]};
     const cudaError_t erb = launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches,
                                                  /*cleanup=*/true);
     if (erb != cudaSuccess) return cuda_fail(h, erb, "store rebuild launch");
@@ -1024,7 +1024,7 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     if (use_graph) {  // one graph per batch shape, replayed
         const GraphKey key{n_ins, n_del, h->push_enabled, h->mode, h->max_iters, h->timing,
                            h->force_rebuild, h->buf_epoch, h->pool_cap[0], h->pool_cap[1],
-                           (const void*)h->d_pool[0], (const void*)h->d_pool[1], h->active};
+                           (const void*)h->d_pool[0], (const void*)h->d_pool[1]};
         if (!h->gexec || !(key == h->gkey)) {
             if (h->gexec) cudaGraphExecDestroy(h->gexec), h->gexec = nullptr;
             cudaGraph_t graph = nullptr;

@@ -54,6 +54,7 @@ struct DevStats {
     unsigned int n_big;        // vertices copied warp-wide in a rebuild
     unsigned int pad0;
     unsigned long long walk_edges; // in-arc walks (SHARED: one per (source group, arc))
+    unsigned long long entries;    // frontier entries processed (SHARED: (vertex, group) rows that pushed)
     // device clock (%globaltimer, ns): POS / NEG phase durations summed over the
     // push launches of a call (one, or one per source wave); restore kernel
     // first-CTA start (atomicMin) and last-CTA end (atomicMax)
@@ -219,6 +220,22 @@ __device__ __forceinline__ unsigned long long l2_keep() {
 __device__ __forceinline__ unsigned long long l2_stream() {
     unsigned long long p;
     asm("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+// policies of the pool (per-edge in-list reads) and slab-descriptor reads (per
+// pushed vertex): 0 = evict_first (streamed), 1 = evict_normal, 2 = evict_last
+#ifndef PPR_POOL_POL
+#define PPR_POOL_POL 0
+#endif
+#ifndef PPR_SLAB_POL
+#define PPR_SLAB_POL 0
+#endif
+template <int K>
+__device__ __forceinline__ unsigned long long l2_pol() {
+    unsigned long long p;
+    if (K == 2) asm("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+    else if (K == 1) asm("createpolicy.fractional.L2::evict_normal.b64 %0, 1.0;" : "=l"(p));
+    else asm("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
     return p;
 }
 __device__ __forceinline__ double atom_add_pol(double* a, double v, unsigned long long pol) {

@@ -222,7 +222,7 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
     const unsigned L = lane(), w = warp();
     const double eps = a.g.eps;
     const uint32_t n = a.g.n;
-    const unsigned long long pol_keep = l2_keep(), pol_stream = l2_stream();
+    const unsigned long long pol_keep = l2_keep(), pol_stream = l2_pol<PPR_POOL_POL>();
     if constexpr (KIND == K_SCAN) {  // fire-and-forget edge walk: no enqueue decisions here
         for (uint32_t cb = w; cb * 32 < E; cb += NW * U) {
             uint32_t v[U], d[U];
@@ -325,7 +325,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             off = q.x;
             len = q.y;
         } else {
-            const ulonglong2 sl = ld_u64x2_pol(&a.g.slab[u], l2_stream());
+            const ulonglong2 sl = ld_u64x2_pol(&a.g.slab[u], l2_pol<PPR_SLAB_POL>());
             off = sl.x;               // Slab::off
             len = (uint32_t)sl.y;     // Slab::len (low word of {len, cap})
         }

@@ -85,6 +85,7 @@ struct MsCtx {
     unsigned long long pushes;     // (source, vertex) self-updates
     unsigned long long edges;      // (source, arc) propagations
     unsigned long long walks;      // (group, arc) walks
+    unsigned long long entries;    // (vertex, group) entries with at least one pushing lane
     uint32_t tiles;                // tiles processed by this CTA (chunk-counter parity)
 };
 
@@ -223,6 +224,7 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
             c.pushes += k;
             c.edges += (unsigned long long)k * len;
             c.walks += len;
+            c.entries++;
         }
     }
     __syncthreads();
@@ -444,7 +446,7 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_co
     __shared__ MsSmem s;
     MsCtx c;
     c.qn = 0;
-    c.pushes = c.edges = c.walks = 0;
+    c.pushes = c.edges = c.walks = c.entries = 0;
     c.tiles = 0;
 #if PPR_MS_WSCAN
     if (threadIdx.x == 0) s.chunk2[0] = s.chunk2[1] = 0;  // ordered by the grid barrier below
@@ -465,17 +467,19 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_co
         atomicAdd(&a.ctl->st.ns_push[0], t1 - t0);
         atomicAdd(&a.ctl->st.ns_push[1], globaltimer_ns() - t1);
     }
-    __shared__ unsigned long long s_red[3];
-    if (threadIdx.x < 3) s_red[threadIdx.x] = 0;
+    __shared__ unsigned long long s_red[4];
+    if (threadIdx.x < 4) s_red[threadIdx.x] = 0;
     __syncthreads();
     if (c.pushes) atomicAdd(&s_red[0], c.pushes);
     if (c.edges) atomicAdd(&s_red[1], c.edges);
     if (c.walks) atomicAdd(&s_red[2], c.walks);
+    if (c.entries) atomicAdd(&s_red[3], c.entries);
     __syncthreads();
     if (threadIdx.x == 0) {
         if (s_red[0]) atomicAdd(&a.ctl->st.pushes, s_red[0]);
         if (s_red[1]) atomicAdd(&a.ctl->st.pushed_edges, s_red[1]);
         if (s_red[2]) atomicAdd(&a.ctl->st.walk_edges, s_red[2]);
+        if (s_red[3]) atomicAdd(&a.ctl->st.entries, s_red[3]);
     }
 }
 

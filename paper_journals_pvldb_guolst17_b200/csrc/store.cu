@@ -100,6 +100,7 @@ __global__ void k_ctl_reset(DevCtl* ctl) {
     ctl->st.arc_delta = 0;
     ctl->st.n_big = 0;
     ctl->st.ns_push[0] = ctl->st.ns_push[1] = 0;
+    ctl->st.walk_edges = ctl->st.entries = 0;
     ctl->st.t_restore[0] = ~0ull;
     ctl->st.t_restore[1] = 0;
 }
@@ -369,10 +370,14 @@ __device__ uint32_t copy_merged_warp(const uint32_t* src, uint32_t* dst, const S
 template <bool PK>
 __device__ __forceinline__ void rebuild_body(const DevGraph& g, const uint64_t* __restrict__ kv,
                                              const BatchBufs& b, const VertexBufs& vb, double slack,
-                                             uint32_t min_cap, uint64_t alt_cap, DevCtl* ctl) {
+                                             uint32_t min_cap, uint64_t cap0, uint64_t cap1,
+                                             DevCtl* ctl) {
     __shared__ uint32_t s_warp[RB_THREADS / 32 + 1];
     __shared__ unsigned long long s_warp64[RB_THREADS / 32 + 1];
     const unsigned act = *(volatile unsigned*)&ctl->st.active_pool;
+    // the spare pool's capacity, read with the device-side active flag (a replayed
+    // batch graph must not bake in the pool that was spare when it was captured)
+    const uint64_t alt_cap = act ? cap0 : cap1;
     const uint32_t* src = act ? g.pool[1] : g.pool[0];
     uint32_t* dst = act ? g.pool[0] : g.pool[1];
     const unsigned lane = threadIdx.x & 31u;
@@ -470,9 +475,10 @@ template <bool PK>
 __global__ void __launch_bounds__(RB_THREADS) k_rebuild(const __grid_constant__ DevGraph g,
                                                         const uint64_t* __restrict__ kv, BatchBufs b,
                                                         VertexBufs vb, double slack, uint32_t min_cap,
-                                                        uint64_t alt_cap, DevCtl* ctl, int cleanup) {
+                                                        uint64_t cap0, uint64_t cap1, DevCtl* ctl,
+                                                        int cleanup) {
     if (*(volatile int*)&ctl->st.err == KERR_OK && *(volatile int*)&ctl->st.rebuild)
-        rebuild_body<PK>(g, kv, b, vb, slack, min_cap, alt_cap, ctl);
+        rebuild_body<PK>(g, kv, b, vb, slack, min_cap, cap0, cap1, ctl);
     if (cleanup) {
         const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
         for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nseg;
@@ -838,10 +844,10 @@ cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t
     VertexBufs vv = vb;
     double slack = sp.slack;
     uint32_t min_cap = sp.min_cap;
-    uint64_t alt_cap = sp.alt_cap;
+    uint64_t cap0 = sp.cap0, cap1 = sp.cap1;
     DevCtl* c = ctl;
     int cl = cleanup ? 1 : 0;
-    void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &alt_cap, &c, &cl};
+    void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &cap0, &cap1, &c, &cl};
     e = cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(RB_THREADS), args, 0, st);
     ++*launches;
     return e;

@@ -42,7 +42,7 @@ struct VertexBufs {
 struct StoreParams {
     double slack;
     uint32_t min_cap;
-    uint64_t alt_cap;  // capacity of the inactive pool (rebuild target)
+    uint64_t cap0, cap1;  // pool capacities; the rebuild targets the one not active on the device
 };
 
 void launch_ctl_reset(DevCtl* ctl, cudaStream_t st, uint32_t* launches);

@@ -50,7 +50,8 @@ class BatchStats(ctypes.Structure):
                 ("d2h_bytes", ctypes.c_uint64), ("ms_total", ctypes.c_float),
                 ("ms_store", ctypes.c_float), ("ms_restore", ctypes.c_float),
                 ("ms_push", ctypes.c_float), ("walk_edges", ctypes.c_uint64),
-                ("ms_push_pos", ctypes.c_float), ("ms_push_neg", ctypes.c_float)]
+                ("ms_push_pos", ctypes.c_float), ("ms_push_neg", ctypes.c_float),
+                ("entries", ctypes.c_uint64)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}

@@ -224,6 +224,25 @@ def test_tiny_config_multi_source_shared(sources):
     _run_stream("tiny", "shared", slides=5, sources=sources, check_every=1)
 
 
+def test_shared_statistics_are_per_call():
+    # walk_edges / entries are the push's own counts for each call (round 1 left
+    # walk_edges accumulating across calls): a call without a push reports 0
+    st, cfg = W.make_stream("tiny")
+    g0s, g0d = st.window()
+    srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 40)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=1e-8, mode="shared")
+    s1 = h.apply_batch(*st.next_batch())
+    assert 0 < s1["walk_edges"] <= s1["pushed_edges"] and 0 < s1["entries"] <= s1["pushes"]
+    s2 = h.apply_batch(*st.next_batch())
+    assert s2["walk_edges"] <= s2["pushed_edges"] and s2["entries"] <= s2["pushes"]
+    h.set_option(ppr.OPT_PUSH, 0)
+    s3 = h.apply_batch(*st.next_batch())
+    assert s3["walk_edges"] == 0 and s3["entries"] == 0 and s3["pushed_edges"] == 0
+    ho = ppr.Ppr(cfg["n"], g0s, g0d, srcs[:1], alpha=0.15, eps=1e-8)
+    so = ho.apply_batch(*st.next_batch())
+    assert so["entries"] == so["pushes"] and so["walk_edges"] == so["pushed_edges"]
+
+
 @pytest.mark.parametrize("wave", [32, 64])
 def test_tiny_config_multi_source_shared_waves(wave):
     # PPR_OPT_WAVE: one push launch per wave of source groups after the shared
@@ -498,6 +517,28 @@ def test_forced_rebuild_path(mode):
         assert stt["rebuilt"] == 1
         o.apply(*b)
         _check_batch_state(h, o, 0, int(srcs[0]), 1e-7, f"rebuild slide {t}")
+
+
+def test_growing_graph_rebuilds_with_replayed_batch_graphs():
+    # insert-only batches of one shape: the batch's CUDA graph is replayed while
+    # rebuilds flip the active pool and the spare pool is regrown to a different
+    # size; the rebuild must check the capacity of the pool that is spare on the
+    # device at replay time (not the one captured)
+    n = 2000
+    src, dst = W.rmat_stream(n, 12_000, seed=21, abc=W.GRAPH500)
+    w0 = 2000
+    (s,) = W.pick_sources(n, src[:w0], dst[:w0], 100, 1)
+    h = ppr.Ppr(n, src[:w0], dst[:w0], [s], alpha=0.15, eps=1e-9, min_cap=1, slack=0.0)
+    o = oracle.Oracle(n, src[:w0], dst[:w0], [s], 0.15, 1e-9)
+    o.push(oracle.SEQ)
+    rebuilt = 0
+    for t in range(10):
+        b = (src[w0 + 1000 * t:w0 + 1000 * (t + 1)], dst[w0 + 1000 * t:w0 + 1000 * (t + 1)], [], [])
+        stt = h.apply_batch(*b)
+        rebuilt += stt["rebuilt"]
+        o.apply(*b)
+        _check_batch_state(h, o, 0, int(s), 1e-9, f"growing slide {t}")
+    assert rebuilt >= 2
 
 
 def test_device_memory_batches():

@@ -124,6 +124,13 @@ typedef struct {
     int l2_persist;      /* persisting L2 access-policy window over R and d_out, passed with each
                             push launch: -1 (default) iff they fit the device's persisting
                             set-aside, 0 never, 1 always */
+    int pool_degrees;    /* in-list (slab pool) entries: 1 = (d_out(u), u) pairs, so the push
+                            reads each divisor d_out(u) with the entry (one dependent random access
+                            per pushed edge fewer), kept exact by a streaming refresh after every
+                            batch's restore; 0 = u32 ids and a d_out gather per pushed edge;
+                            -1 (default): pairs iff R + d_out exceed the persisting L2 set-aside
+                            (DRAM-resident: Twitter shape push -28%; L2-resident: LJ shape +6%).
+                            1 with layout = PPR_LAYOUT_PACKED: PPR_EINVAL. */
 } ppr_opts;
 
 enum { PPR_LAYOUT_ARRAYS = 0, PPR_LAYOUT_PACKED = 1 };

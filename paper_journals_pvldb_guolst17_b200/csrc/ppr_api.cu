@@ -81,7 +81,8 @@ struct ppr_ctx {
     float l2_hit = 0.f;
     uint32_t* d_dout = nullptr;  // structure-of-arrays layout (S > 1)
     Slab* d_slab = nullptr;
-    uint32_t* d_pool[2] = {nullptr, nullptr};
+    PoolEnt* d_pool[2] = {nullptr, nullptr};  // slab pools (entries: PoolEnt if pool_wide, else u32)
+    bool pool_wide = false;                   // ppr_opts.pool_degrees (ppr_internal.cuh PoolEnt)
     double* d_P = nullptr;
     double* d_R = nullptr;
     uint32_t* d_sources = nullptr;  // internal ids
@@ -213,6 +214,9 @@ void dfree(ppr_ctx* h, T*& p, uint64_t count) {
     p = nullptr;
 }
 
+// PoolEnt-sized words backing a pool of `cap` entries (4 or 8 bytes each)
+uint64_t pool_words(const ppr_ctx* h, uint64_t cap) { return h->pool_wide ? cap : (cap + 1) / 2; }
+
 DevGraph graph_of(const ppr_ctx* h) {
     DevGraph g;
     g.n = h->n;
@@ -223,6 +227,7 @@ DevGraph graph_of(const ppr_ctx* h) {
     g.slab = h->d_slab;
     g.pool[0] = h->d_pool[0];
     g.pool[1] = h->d_pool[1];
+    g.pool_wide = h->pool_wide ? 1u : 0u;
     g.P = h->d_P;
     g.R = h->d_R;
     g.sources = h->d_sources;
@@ -300,15 +305,16 @@ ppr_status ensure_alt_pool(ppr_ctx* h, uint64_t new_arcs) {
     if (h->pool_cap[alt] >= need) return PPR_OK;
     cudaError_t e = cudaStreamSynchronize(h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, "ensure_alt_pool sync");
-    dfree(h, h->d_pool[alt], h->pool_cap[alt]);
+    dfree(h, h->d_pool[alt], pool_words(h, h->pool_cap[alt]));
     h->pool_cap[alt] = 0;
     h->buf_epoch++;
     uint64_t cap = need + need / 4;
-    if (dalloc(h, &h->d_pool[alt], cap) != cudaSuccess) {
+    if (dalloc(h, &h->d_pool[alt], pool_words(h, cap)) != cudaSuccess) {
         set_err(h, "out of device memory for the rebuild pool (%llu entries)",
                 (unsigned long long)cap);
         return PPR_ENOMEM;
     }
+    cudaMemsetAsync(h->d_pool[alt], 0xFF, sizeof(PoolEnt) * pool_words(h, cap), h->st);  // empty slots
     h->pool_cap[alt] = cap;
     return PPR_OK;
 }
@@ -439,8 +445,8 @@ void destroy_all(ppr_ctx* h) {
     }
     dfree(h, h->d_dout, h->n);
     dfree(h, h->d_slab, h->n);
-    dfree(h, h->d_pool[0], h->pool_cap[0]);
-    dfree(h, h->d_pool[1], h->pool_cap[1]);
+    dfree(h, h->d_pool[0], pool_words(h, h->pool_cap[0]));
+    dfree(h, h->d_pool[1], pool_words(h, h->pool_cap[1]));
     dfree(h, h->d_P, (uint64_t)h->S * h->n);
     dfree(h, h->d_R, (uint64_t)h->S * h->n);
     dfree(h, h->d_sources, h->S);
@@ -475,7 +481,10 @@ void destroy_all(ppr_ctx* h) {
     h->st = nullptr;
 }
 
-constexpr uint64_t kRingTailDefault = 16384;  // entries
+#ifndef PPR_RING_TAIL_DEFAULT
+#define PPR_RING_TAIL_DEFAULT 16384
+#endif
+constexpr uint64_t kRingTailDefault = PPR_RING_TAIL_DEFAULT;  // entries
 bool ring_fits(const ppr_ctx* h) { return (uint64_t)h->S * h->n <= (1ull << 27); }
 
 ppr_status ensure_ring(ppr_ctx* h) {
@@ -613,7 +622,7 @@ ppr_status enqueue_batch(ppr_ctx* h, const uint32_t* is, const uint32_t* id, uin
     // the reset of the v -> segment map
     StoreParams sp{h->slack, h->min_cap, h->pool_cap[0], h->pool_cap[1]};
     const cudaError_t erb = launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches,
-                                                 /*cleanup=*/true);
+                                                 /*finish=*/true);
     if (erb != cudaSuccess) return cuda_fail(h, erb, "store rebuild launch");
     *launches_out = launches;
     return PPR_OK;
@@ -672,9 +681,11 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     o.relabel = -1;
     o.layout = PPR_LAYOUT_ARRAYS;
     o.l2_persist = -1;
+    o.pool_degrees = -1;
     if (opts) o = *opts;
     if (o.mode < PPR_MODE_OPT || o.mode > PPR_MODE_SORTAGG || !(o.slack >= 0.0) ||
-        o.min_cap == 0 || (o.layout != PPR_LAYOUT_ARRAYS && o.layout != PPR_LAYOUT_PACKED))
+        o.min_cap == 0 || (o.layout != PPR_LAYOUT_ARRAYS && o.layout != PPR_LAYOUT_PACKED) ||
+        o.pool_degrees < -1 || o.pool_degrees > 1)
         return PPR_EINVAL;
 
     ppr_ctx* h = new (std::nothrow) ppr_ctx();
@@ -751,6 +762,9 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         cudaDeviceGetAttribute(&maxp, cudaDevAttrMaxPersistingL2CacheSize, h->device);
         cudaDeviceGetAttribute(&maxw, cudaDevAttrMaxAccessPolicyWindowSize, h->device);
         const bool want = o.l2_persist > 0 || (o.l2_persist < 0 && h->hot_bytes <= (uint64_t)maxp);
+        // degrees cached in the pool entries iff R + d_out do not fit the persisting
+        // set-aside (DRAM-resident gathers; ppr_internal.cuh PoolEnt)
+        h->pool_wide = o.pool_degrees > 0 || (o.pool_degrees < 0 && h->hot_bytes > (uint64_t)maxp);
         if (want && maxp > 0 && maxw > 0) {
             // the window travels with each push launch (launch attribute); the
             // caller's stream is left alone.  The device-wide set-aside is raised
@@ -764,6 +778,11 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
                 fprintf(stderr, "ppr: L2 window %zu B of %llu hot (max window %d, max set-aside %d), hit ratio %.3f\n",
                         win, (unsigned long long)h->hot_bytes, maxw, maxp, h->l2_hit);
         }
+    }
+    if (packed && o.pool_degrees > 0) {  // the packed records keep u32 in-list entries
+        destroy_all(h);
+        delete h;
+        return PPR_EINVAL;
     }
     ok = ok &&
               dalloc(h, &h->d_sources, h->S) == cudaSuccess &&
@@ -865,14 +884,18 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         if (cap < total + 1024) cap = total + 1024;
         h->pool_cap[0] = h->pool_cap[1] = cap;
     }
-    if (dalloc(h, &h->d_pool[0], h->pool_cap[0]) != cudaSuccess ||
-        dalloc(h, &h->d_pool[1], h->pool_cap[0]) != cudaSuccess) {
+    if (dalloc(h, &h->d_pool[0], pool_words(h, h->pool_cap[0])) != cudaSuccess ||
+        dalloc(h, &h->d_pool[1], pool_words(h, h->pool_cap[1])) != cudaSuccess) {
         dfree(h, d_src, g->m);
         dfree(h, d_dst, g->m);
         destroy_all(h);
         delete h;
         return PPR_ENOMEM;
     }
+    // every slot starts POOL_EMPTY (slab slack stays empty; the degree refresh streams the pool)
+    cudaMemsetAsync(h->d_pool[0], 0xFF, sizeof(PoolEnt) * pool_words(h, h->pool_cap[0]), st);
+    cudaMemsetAsync(h->d_pool[1], 0xFF, sizeof(PoolEnt) * pool_words(h, h->pool_cap[1]), st);
+    cudaMemcpyAsync(&h->d_ctl->st.pool_extent, &total, sizeof total, cudaMemcpyHostToDevice, st);
     dg = graph_of(h);
     launch_build_fill(d_src, d_dst, g->m, h->undirected, dg, h->vb, st, &launches);
     launch_init_state(dg, st, &launches);

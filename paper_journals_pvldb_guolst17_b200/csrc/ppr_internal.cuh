@@ -55,6 +55,7 @@ struct DevStats {
     unsigned int pad0;
     unsigned long long walk_edges; // in-arc walks (SHARED: one per (source group, arc))
     unsigned long long entries;    // frontier entries processed (SHARED: (vertex, group) rows that pushed)
+    unsigned long long pool_extent; // slots [0, extent) of the active pool hold slabs (build / rebuild)
     // device clock (%globaltimer, ns): POS / NEG phase durations summed over the
     // push launches of a call (one, or one per source wave); restore kernel
     // first-CTA start (atomicMin) and last-CTA end (atomicMax)
@@ -89,6 +90,28 @@ struct DevCtl {
     DevStats st;
 };
 
+// Slab-pool entries of N_in(v), two formats chosen per handle (DevGraph::pool_wide):
+//  * wide (PoolEnt): the in-neighbour u AND its current out-degree,
+//    (d_out(u) << 32) | u.  The push reads the divisor d(u) of Alg 3 line 19 with
+//    the in-list entry itself -- one dependent random access per pushed edge
+//    fewer than a separate d_out[u] gather, which matters when d_out is
+//    DRAM-resident (Twitter shape: push 96 -> 69 ms per batch).  The store keeps
+//    the cached degrees exact: after every batch's restore has updated d_out, the
+//    last store launch streams the active pool and rewrites the entries whose
+//    degree changed.  Unused slots (slab slack) hold POOL_EMPTY so that stream
+//    needs no slab descriptors.
+//  * narrow (u32 ids, d_out gathered per edge): when R and d_out are L2-resident
+//    the gather is cheap and the refresh stream would cost more than it saves
+//    (LJ shape: 3.30 vs 3.49 ms per batch).
+// Vertex ids are < 2^32 - 1 (ppr_create), so u = 0xFFFFFFFF marks an empty slot.
+using PoolEnt = unsigned long long;
+constexpr PoolEnt POOL_EMPTY = ~0ull;
+__host__ __device__ __forceinline__ uint32_t pe_v(PoolEnt e) { return (uint32_t)e; }
+__host__ __device__ __forceinline__ uint32_t pe_d(PoolEnt e) { return (uint32_t)(e >> 32); }
+__host__ __device__ __forceinline__ PoolEnt pe_make(uint32_t v, uint32_t d) {
+    return ((PoolEnt)d << 32) | v;
+}
+
 struct DevGraph {
     uint32_t n;
     uint32_t S;
@@ -96,7 +119,8 @@ struct DevGraph {
     double eps;
     uint32_t* dout;
     Slab* slab;
-    uint32_t* pool[2];
+    PoolEnt* pool[2];         // slab pools (one active, one rebuild target); u32 entries if !pool_wide
+    uint32_t pool_wide;       // 1: PoolEnt entries carry d_out; 0: u32 in-neighbour ids
     double* P;
     double* R;
     const uint32_t* sources;  // [S]
@@ -149,6 +173,27 @@ __device__ __forceinline__ void put_slab(const DevGraph& g, uint64_t v, const Sl
     } else {
         g.slab[v] = s;
     }
+}
+
+// ------------------------------------------------------------------ pool entries (either format)
+
+__device__ __forceinline__ uint32_t pool_id(const DevGraph& g, const PoolEnt* pool, uint64_t i) {
+    return g.pool_wide ? pe_v(pool[i]) : reinterpret_cast<const uint32_t*>(pool)[i];
+}
+__device__ __forceinline__ void pool_copy(const DevGraph& g, PoolEnt* dst, uint64_t j,
+                                          const PoolEnt* src, uint64_t i) {
+    if (g.pool_wide) dst[j] = src[i];
+    else reinterpret_cast<uint32_t*>(dst)[j] = reinterpret_cast<const uint32_t*>(src)[i];
+}
+// d: d_out(v) for the wide format (0 = "not yet known", set by the degree refresh)
+__device__ __forceinline__ void pool_put(const DevGraph& g, PoolEnt* pool, uint64_t i, uint32_t v,
+                                         uint32_t d) {
+    if (g.pool_wide) pool[i] = pe_make(v, d);
+    else reinterpret_cast<uint32_t*>(pool)[i] = v;
+}
+__device__ __forceinline__ void pool_clear(const DevGraph& g, PoolEnt* pool, uint64_t i) {
+    if (g.pool_wide) pool[i] = POOL_EMPTY;
+    else reinterpret_cast<uint32_t*>(pool)[i] = 0xFFFFFFFFu;
 }
 
 // ------------------------------------------------------------------ helpers
@@ -259,29 +304,14 @@ __device__ __forceinline__ uint32_t ld_u32_pol(const uint32_t* a, unsigned long 
     asm volatile("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
     return r;
 }
-// the push's two per-edge loads: the pool entry is streamed (read once per
-// walk: PPR_L1_POOL_NA=1 keeps it out of L1), d_out(v) is re-read for every
-// pushed in-arc of v (PPR_L1_DOUT_EL=1 asks L1 to keep it)
-#ifndef PPR_L1_POOL_NA
-#define PPR_L1_POOL_NA 0
-#endif
-#ifndef PPR_L1_DOUT_EL
-#define PPR_L1_DOUT_EL 0
-#endif
-__device__ __forceinline__ uint32_t ld_pool(const uint32_t* a, unsigned long long pol) {
+__device__ __forceinline__ uint32_t ld_u32_nc_pol(const uint32_t* a, unsigned long long pol) {
     uint32_t r;
-    if (PPR_L1_POOL_NA)
-        asm volatile("ld.global.nc.L1::no_allocate.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
-    else
-        asm volatile("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
+    asm volatile("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
     return r;
 }
-__device__ __forceinline__ uint32_t ld_dout(const uint32_t* a, unsigned long long pol) {
-    uint32_t r;
-    if (PPR_L1_DOUT_EL)
-        asm volatile("ld.global.nc.L1::evict_last.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
-    else
-        asm volatile("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(r) : "l"(a), "l"(pol));
+__device__ __forceinline__ PoolEnt ld_pool_ent(const PoolEnt* a, unsigned long long pol) {
+    PoolEnt r;
+    asm volatile("ld.global.nc.L2::cache_hint.u64 %0, [%1], %2;" : "=l"(r) : "l"(a), "l"(pol));
     return r;
 }
 __device__ __forceinline__ ulonglong2 ld_u64x2_pol(const void* a, unsigned long long pol) {

@@ -44,6 +44,12 @@ namespace ppr {
 
 namespace {
 
+// vertex layout / pool format of a push instantiation (template parameter LAY):
+// arrays with u32 in-list entries, packed VRec records, arrays with PoolEnt entries
+// that carry d_out (ppr_internal.cuh) -- compile-time, so the hot loop of each
+// format has no branch and no registers for the other
+constexpr int LAY_ARRAYS = 0, LAY_PACKED = 1, LAY_WIDE = 2;
+
 constexpr int PT = PUSH_THREADS;
 constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_PUSH_U
@@ -89,7 +95,7 @@ struct Smem {
 
 
 struct Ctx {
-    const uint32_t* pool;
+    const PoolEnt* pool;
     unsigned long long* Fout;
     unsigned long long* cnt_out;
     unsigned long long* trace_edges;  // this round's edge counter (trace mode) or null
@@ -192,7 +198,7 @@ __device__ __forceinline__ int owner_of(const uint32_t* scan, uint32_t e, int to
 
 // ---------------------------------------------------------------- CTA tile
 
-template <bool POS, int KIND, bool PK>
+template <bool POS, int KIND, int LAY>
 __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
                                           unsigned long long ent, uint64_t idx, uint32_t T,
                                           int top);
@@ -200,14 +206,27 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
 // Processes the T entries Fin[base_idx .. base_idx+T) (thread i = entry i):
 // neighbour propagation of every pushed entry and, for K_OPT, the fused
 // self-update.  Must be called by all threads of the CTA.
-template <bool POS, int KIND, bool PK>
+template <bool POS, int KIND, int LAY>
 __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
                                          const unsigned long long* Fin, uint64_t C,
                                          uint64_t base_idx, uint32_t T, int top) {
     const uint64_t idx = base_idx + threadIdx.x;
     const bool valid = threadIdx.x < T && idx < C;
     const unsigned long long ent = valid ? __ldcg(&Fin[idx]) : 0ull;
-    tile_body<POS, KIND, PK>(s, c, a, valid, ent, idx, T, top);
+    tile_body<POS, KIND, LAY>(s, c, a, valid, ent, idx, T, top);
+}
+
+// in-list entry i of the active pool: v, and d_out(v) for the wide format
+template <int LAY>
+__device__ __forceinline__ void load_entry(const PoolEnt* pool, uint64_t i, unsigned long long pol,
+                                           uint32_t& v, uint32_t& d) {
+    if constexpr (LAY == LAY_WIDE) {
+        const PoolEnt pe = ld_pool_ent(&pool[i], pol);
+        v = pe_v(pe);
+        d = pe_d(pe);
+    } else {
+        v = ld_u32_nc_pol(reinterpret_cast<const uint32_t*>(pool) + i, pol);
+    }
 }
 
 // Walks the E edges of one prepared tile (scan/off/w/sid, the entries' in-lists
@@ -216,7 +235,7 @@ __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
 // search in the prefix, and runs the chain pool entry -> d_out(v) ->
 // atomicAdd(R(v), (1-a) r_u / d(v)) (Alg 3 lines 17-20 / Alg 4 lines 11-17).
 // All U atomics of a step are issued before any result is consumed.
-template <bool POS, int KIND, bool PK>
+template <bool POS, int KIND, int LAY>
 __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, const TileArrays& t,
                                            uint32_t E, int top, unsigned int* chunkp) {
     const unsigned L = lane(), w = warp();
@@ -232,19 +251,22 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
                 const uint32_t e = (cb + NW * k) * 32 + L;
                 j[k] = -1;
                 v[k] = 0;
+                d[k] = 1;
                 if (e < E) {
                     j[k] = owner_of(t.scan, e, top);
-                    v[k] = ld_pool(&c.pool[t.off[j[k]] + (e - t.scan[j[k]])], pol_stream);
+                    load_entry<LAY>(c.pool, t.off[j[k]] + (e - t.scan[j[k]]), pol_stream, v[k], d[k]);
                 }
             }
+            if constexpr (LAY != LAY_WIDE) {
 #pragma unroll
-            for (int k = 0; k < U; k++)
-                d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_dout(&a.g.dout[v[k]], pol_keep));
+                for (int k = 0; k < U; k++)
+                    if (j[k] >= 0) d[k] = (LAY == LAY_PACKED) ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_nc_pol(&a.g.dout[v[k]], pol_keep);
+            }
 #pragma unroll
             for (int k = 0; k < U; k++) {
                 if (j[k] >= 0) {
                     const uint32_t sj = t.sid[j[k]];
-                    red_add_pol(Rp<PK>(a.g, sj, v[k]), __ddiv_rn(t.w[j[k]], (double)d[k]), pol_keep);
+                    red_add_pol(Rp<(LAY == LAY_PACKED)>(a.g, sj, v[k]), __ddiv_rn(t.w[j[k]], (double)d[k]), pol_keep);
                     mark_bit(a.bitmap, (size_t)v[k] * a.g.S + sj);
                 }
             }
@@ -258,22 +280,25 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
         cb = __shfl_sync(0xffffffffu, cb, 0);
         if (cb * 32 >= E) break;
         ensure_room(s, c, 32 * U);
-        uint32_t v[U];
+        uint32_t v[U], d[U];
         int j[U];
 #pragma unroll
         for (int k = 0; k < U; k++) {
             const uint32_t e = (cb + k) * 32 + L;
             j[k] = -1;
             v[k] = 0;
+            d[k] = 1;
             if (e < E) {
                 j[k] = owner_of(t.scan, e, top);
-                v[k] = ld_pool(&c.pool[t.off[j[k]] + (e - t.scan[j[k]])], pol_stream);
+                // wide pool: one 8-byte load gives v and d_out(v) (ppr_internal.cuh PoolEnt)
+                load_entry<LAY>(c.pool, t.off[j[k]] + (e - t.scan[j[k]]), pol_stream, v[k], d[k]);
             }
         }
-        uint32_t d[U];
+        if constexpr (LAY != LAY_WIDE) {  // narrow pool: gather d_out(v), all U loads in flight
 #pragma unroll
-        for (int k = 0; k < U; k++)
-            d[k] = j[k] < 0 ? 1u : (PK ? __ldcg(&a.g.rec[v[k]].dout) : ld_dout(&a.g.dout[v[k]], pol_keep));
+            for (int k = 0; k < U; k++)
+                if (j[k] >= 0) d[k] = (LAY == LAY_PACKED) ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_nc_pol(&a.g.dout[v[k]], pol_keep);
+        }
         double incr[U], pre[U];
         uint32_t sj[U];
 #pragma unroll
@@ -281,7 +306,7 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
             if (j[k] >= 0) {
                 sj[k] = t.sid[j[k]];
                 incr[k] = __ddiv_rn(t.w[j[k]], (double)d[k]);
-                pre[k] = atom_add_pol(Rp<PK>(a.g, sj[k], v[k]), incr[k], pol_keep);
+                pre[k] = atom_add_pol(Rp<(LAY == LAY_PACKED)>(a.g, sj[k], v[k]), incr[k], pol_keep);
             }
         }
 #pragma unroll
@@ -306,13 +331,13 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
 // The tile's work once thread i holds entry i (valid, ent; idx indexes W):
 // the entry's residual read / self-update, the CTA-wide prefix of the
 // pushed entries' in-degrees, then the edge walk by all warps.
-template <bool POS, int KIND, bool PK>
+template <bool POS, int KIND, int LAY>
 __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
                                           unsigned long long ent, uint64_t idx, uint32_t T,
                                           int top) {
     const double eps = a.g.eps, alpha = a.g.alpha;
     const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
-    double* ru = Rp<PK>(a.g, sidx, u);
+    double* ru = Rp<(LAY == LAY_PACKED)>(a.g, sidx, u);
     double r = 0.0;
     bool push = false;
     // the slab descriptor depends only on u: issued before (and overlapping)
@@ -320,7 +345,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     uint32_t len = 0;
     unsigned long long off = 0;
     if (valid) {
-        if (PK) {  // {off, len} of the vertex record (same sector as R(u), P(u))
+        if ((LAY == LAY_PACKED)) {  // {off, len} of the vertex record (same sector as R(u), P(u))
             const uint2 q = __ldcg(reinterpret_cast<const uint2*>(&a.g.rec[u].off));
             off = q.x;
             len = q.y;
@@ -337,7 +362,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
         // (DESIGN.md K-PUSH).
         r = valid ? atom_exch_f64_pol(ru, 0.0, l2_keep()) : 0.0;
         push = valid && r != 0.0;
-        if (push) red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
+        if (push) red_add_pol(Pp<(LAY == LAY_PACKED)>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
     } else if (KIND == K_EAGER || KIND == K_SCAN) {
         r = valid ? ld_relaxed_f64(ru) : 0.0;  // Alg 4 line 10: the current R(u)
         push = valid && push_cond<POS>(r, eps);
@@ -348,7 +373,7 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     }
     if (KIND == K_SCAN && push) {  // self-update: no result needed; u is re-tested at the scan
         red_add_pol(ru, -r, l2_keep());
-        red_add_pol(Pp<PK>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
+        red_add_pol(Pp<(LAY == LAY_PACKED)>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
         mark_bit(a.bitmap, (size_t)u * a.g.S + sidx);
     }
     if (!push) len = 0;
@@ -369,12 +394,12 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
         c.edges += E;
         if (c.trace_edges && E) atomicAdd(c.trace_edges, (unsigned long long)E);
     }
-    walk_edges<POS, KIND, PK>(s, c, a, s.t, E, top, &s.chunk);
+    walk_edges<POS, KIND, LAY>(s, c, a, s.t, E, top, &s.chunk);
 }
 
 // Every CTA takes tiles of T entries: its first tile statically, the rest by
 // one atomic claim each, until C is covered.
-template <bool POS, int KIND, bool PK>
+template <bool POS, int KIND, int LAY>
 __device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a, const unsigned long long* Fin,
                               uint64_t C, unsigned long long* tc) {
     uint64_t per = (C + gridDim.x - 1) / gridDim.x;
@@ -387,7 +412,7 @@ __device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a
     uint64_t t = blockIdx.x;
     while (t < ntiles) {
         if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark = globaltimer_ns();
-        cta_tile<POS, KIND, PK>(s, c, a, Fin, C, t * T, T, top);
+        cta_tile<POS, KIND, LAY>(s, c, a, Fin, C, t * T, T, top);
         if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark2 = globaltimer_ns();
         if (ntiles <= gridDim.x) break;  // every tile was assigned statically
         if (threadIdx.x == 0) s.next = atomicAdd(tc, 1ull) + gridDim.x;
@@ -402,7 +427,7 @@ __device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a
 // ---------------------------------------------------------------- Alg 3 / Eager sessions
 
 // self-update session of Alg 3 (lines 13-16): w = R(u), P(u) += a w, R(u) = 0
-template <bool PK>
+template <int LAY>
 __device__ __forceinline__ void session_snapshot(Ctx& c, const PushArgs& a, const unsigned long long* Fin,
                                  uint64_t C, bool bitmap) {
     const double alpha = a.g.alpha;
@@ -410,8 +435,8 @@ __device__ __forceinline__ void session_snapshot(Ctx& c, const PushArgs& a, cons
          idx += (uint64_t)gridDim.x * PT) {
         const unsigned long long ent = __ldcg(&Fin[idx]);
         const size_t i = (size_t)(ent >> 32) * a.g.n + (uint32_t)ent;
-        double* rp = Rp<PK>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent);
-        double* pp = Pp<PK>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent);
+        double* rp = Rp<(LAY == LAY_PACKED)>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent);
+        double* pp = Pp<(LAY == LAY_PACKED)>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent);
         const double w = __ldcg(rp);
         __stcg(pp, __dadd_rn(__ldcg(pp), __dmul_rn(alpha, w)));
         __stcg(rp, 0.0);
@@ -422,7 +447,7 @@ __device__ __forceinline__ void session_snapshot(Ctx& c, const PushArgs& a, cons
 }
 
 // Eager: self-update with the r_u recorded during propagation (Alg 4 lines 19-23)
-template <bool POS, bool PK>
+template <bool POS, int LAY>
 __device__ __forceinline__ void session_eager_self(Smem& s, Ctx& c, const PushArgs& a,
                                    const unsigned long long* Fin, uint64_t C) {
     const double eps = a.g.eps, alpha = a.g.alpha;
@@ -436,9 +461,9 @@ __device__ __forceinline__ void session_eager_self(Smem& s, Ctx& c, const PushAr
             const double r = __ldcg(&a.W[idx]);
             if (r != 0.0) {
                 const size_t i = (size_t)(ent >> 32) * a.g.n + (uint32_t)ent;
-                const double old = atomicAdd(Rp<PK>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent), -r);
+                const double old = atomicAdd(Rp<(LAY == LAY_PACKED)>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent), -r);
                 const double cur = __dadd_rn(old, -r);
-                atomicAdd(Pp<PK>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent), __dmul_rn(alpha, r));
+                atomicAdd(Pp<(LAY == LAY_PACKED)>(a.g, (uint32_t)(ent >> 32), (uint32_t)ent), __dmul_rn(alpha, r));
                 c.pushes++;
                 enq = push_cond<POS>(cur, eps) && test_and_set(a.bitmap, i);
             }
@@ -468,7 +493,7 @@ __device__ __forceinline__ void clear_frontier_bits(Ctx& c, const PushArgs& a, c
 // emitted frontier is exactly {(s,v) : pushCond(R_s(v))} (Alg 3 line 1,
 // restricted to the vertices the round touched) and is sorted by vertex
 // within each warp's word range.
-template <bool POS, bool PK>
+template <bool POS, int LAY>
 __device__ __forceinline__ void scan_bitmap(Smem& s, Ctx& c, const PushArgs& a) {
     const double eps = a.g.eps;
     const uint64_t nbits = (uint64_t)a.g.S * a.g.n;
@@ -487,7 +512,7 @@ __device__ __forceinline__ void scan_bitmap(Smem& s, Ctx& c, const PushArgs& a) 
                 word &= word - 1;
                 const uint64_t bit = wi * 32 + b;
                 const uint32_t v = (uint32_t)(bit / a.g.S), sidx = (uint32_t)(bit % a.g.S);
-                enq = push_cond<POS>(__ldcg(Rp<PK>(a.g, sidx, v)), eps);
+                enq = push_cond<POS>(__ldcg(Rp<(LAY == LAY_PACKED)>(a.g, sidx, v)), eps);
                 ent = ((unsigned long long)sidx << 32) | v;
             }
             ensure_room(s, c, 32);
@@ -498,7 +523,7 @@ __device__ __forceinline__ void scan_bitmap(Smem& s, Ctx& c, const PushArgs& a) 
 
 // ---------------------------------------------------------------- seeding
 
-template <bool POS, bool PK>
+template <bool POS, int LAY>
 __device__ __forceinline__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
     const double eps = a.g.eps;
     const uint64_t stride = (uint64_t)gridDim.x * PT;
@@ -528,7 +553,7 @@ __device__ __forceinline__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
                 v = (uint32_t)ent;
             }
             ent = ((unsigned long long)sidx << 32) | v;
-            enq = push_cond<POS>(__ldcg(Rp<PK>(a.g, sidx, v)), eps);
+            enq = push_cond<POS>(__ldcg(Rp<(LAY == LAY_PACKED)>(a.g, sidx, v)), eps);
         }
         ensure_room(s, c, 32);
         warp_enqueue(s, c, enq, ent);
@@ -543,11 +568,11 @@ __device__ __forceinline__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
 // for a few thousand pushes), so the rest of the phase runs on the
 // asynchronous ring schedule instead (the same operations without round
 // barriers; any push order is valid, Lemma 1; DESIGN.md K-ASYNC).
-template <bool POS, bool PK>
+template <bool POS, int LAY>
 __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, unsigned long long* head,
                                            unsigned long long* tail, unsigned long long* done);
 
-template <bool POS, bool PK>
+template <bool POS, int LAY>
 __device__ __forceinline__ void hybrid_tail(Smem& s, Ctx& c, const PushArgs& a,
                                             const unsigned long long* Fin, uint64_t C) {
     DevCtl* ctl = a.ctl;
@@ -561,7 +586,7 @@ __device__ __forceinline__ void hybrid_tail(Smem& s, Ctx& c, const PushArgs& a,
     c.Fout = a.ring;
     c.cnt_out = tail;
     c.ring_cap = a.ring_cap;
-    async_loop<POS, PK>(s, c, a, head, tail, done);
+    async_loop<POS, LAY>(s, c, a, head, tail, done);
     c.ring_cap = 0;
     grid_sync(ctl);
     if (blockIdx.x == 0 && threadIdx.x == 0) *head = *tail = *done = 0;
@@ -569,14 +594,14 @@ __device__ __forceinline__ void hybrid_tail(Smem& s, Ctx& c, const PushArgs& a,
 
 // ---------------------------------------------------------------- phase driver
 
-template <int MODE, bool POS, bool PK>
+template <int MODE, bool POS, int LAY>
 __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, unsigned& it) {
     DevCtl* ctl = a.ctl;
     const int ph = POS ? 0 : 1;
     // seed into F[it%2] / fcount[it%3]; both that and the next counter are 0 here
     c.Fout = a.F[it & 1];
     c.cnt_out = &ctl->fcount[it % 3].v;
-    seed_phase<POS, PK>(s, c, a);
+    seed_phase<POS, LAY>(s, c, a);
     block_flush(s, c);
     grid_sync(ctl);
     uint32_t pit = 0;
@@ -606,7 +631,7 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
         // once the frontier is past its peak and at most hyb_thresh entries
         if (MODE == M_OPT && a.ring && !a.max_iters &&
             (a.hyb_all || (pit > 0 && C <= a.hyb_thresh && C <= Cprev))) {
-            hybrid_tail<POS, PK>(s, c, a, Fin, C);  // the phase ends on the ring
+            hybrid_tail<POS, LAY>(s, c, a, Fin, C);  // the phase ends on the ring
             it++;
             C = 0;
             break;
@@ -616,24 +641,24 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
         unsigned long long* tc = &ctl->tilectr[it % 3].v;
         const unsigned long long t0 = (kTimeSplit && a.trace) ? globaltimer_ns() : 0;
         if (MODE == M_OPT) {
-            propagate_all<POS, K_OPT, PK>(s, c, a, Fin, C, tc);
+            propagate_all<POS, K_OPT, LAY>(s, c, a, Fin, C, tc);
         } else if (MODE == M_SCAN) {
-            propagate_all<POS, K_SCAN, PK>(s, c, a, Fin, C, tc);
+            propagate_all<POS, K_SCAN, LAY>(s, c, a, Fin, C, tc);
             grid_sync(ctl);  // every reduction of the round has landed
-            scan_bitmap<POS, PK>(s, c, a);
+            scan_bitmap<POS, LAY>(s, c, a);
         } else if (MODE == M_VAN || MODE == M_DUP) {
-            session_snapshot<PK>(c, a, Fin, C, MODE == M_VAN);
+            session_snapshot<LAY>(c, a, Fin, C, MODE == M_VAN);
             grid_sync(ctl);
             if (MODE == M_VAN)
-                propagate_all<POS, K_VAN, PK>(s, c, a, Fin, C, tc);
+                propagate_all<POS, K_VAN, LAY>(s, c, a, Fin, C, tc);
             else
-                propagate_all<POS, K_DUP, PK>(s, c, a, Fin, C, tc);
+                propagate_all<POS, K_DUP, LAY>(s, c, a, Fin, C, tc);
         } else {  // M_EAGER
             clear_frontier_bits(c, a, Fin, C);
             grid_sync(ctl);
-            propagate_all<POS, K_EAGER, PK>(s, c, a, Fin, C, tc);
+            propagate_all<POS, K_EAGER, LAY>(s, c, a, Fin, C, tc);
             grid_sync(ctl);
-            session_eager_self<POS, PK>(s, c, a, Fin, C);
+            session_eager_self<POS, LAY>(s, c, a, Fin, C);
         }
         const unsigned long long t1 = (kTimeSplit && a.trace) ? globaltimer_ns() : 0;
         block_flush(s, c);
@@ -660,7 +685,7 @@ __device__ __forceinline__ void run_phase(Smem& s, Ctx& c, const PushArgs& a, un
     grid_sync(ctl);
 }
 
-template <int MODE, bool PK>
+template <int MODE, int LAY>
 __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_constant__ PushArgs a) {
     __shared__ Smem s;
     Ctx c;
@@ -680,9 +705,9 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push(const __grid_const
     const bool stamp = blockIdx.x == 0 && threadIdx.x == 0;
     const unsigned long long t0 = stamp ? globaltimer_ns() : 0;
     unsigned it = 0;
-    if (a.phases & 1) run_phase<MODE, true, PK>(s, c, a, it);
+    if (a.phases & 1) run_phase<MODE, true, LAY>(s, c, a, it);
     const unsigned long long t1 = stamp ? globaltimer_ns() : 0;  // run_phase ends with a grid barrier
-    if (a.phases & 2) run_phase<MODE, false, PK>(s, c, a, it);
+    if (a.phases & 2) run_phase<MODE, false, LAY>(s, c, a, it);
     if (stamp) {  // phase durations, summed over launches (source waves)
         atomicAdd(&a.ctl->st.ns_push[0], t1 - t0);
         atomicAdd(&a.ctl->st.ns_push[1], globaltimer_ns() - t1);
@@ -757,7 +782,7 @@ inline cudaError_t coop_launch(const void* fn, int grid, const PushArgs& a, cuda
 // The ring loop: CTAs claim chunks of queued entries and process each chunk
 // as a tile until done == tail.  Entry: the ring holds the seeds, tail = their
 // count, head = done = 0, c.Fout/c.cnt_out/c.ring_cap point at the ring.
-template <bool POS, bool PK>
+template <bool POS, int LAY>
 __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, unsigned long long* head,
                                            unsigned long long* tail, unsigned long long* done) {
     __shared__ unsigned long long s_h, s_k;
@@ -816,7 +841,7 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
         }
         int top = 1;
         while (top * 2 < (int)k) top <<= 1;
-        tile_body<POS, K_OPT, PK>(s, c, a, valid, ent, 0, k, top);
+        tile_body<POS, K_OPT, LAY>(s, c, a, valid, ent, 0, k, top);
         block_flush(s, c);  // this tile's children reach `tail` ...
         if (threadIdx.x == 0) {  // ... before it counts as done (release: tail and the slots first)
             __threadfence();
@@ -825,7 +850,7 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
     }
 }
 
-template <bool POS, bool PK>
+template <bool POS, int LAY>
 __device__ __forceinline__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) {
     DevCtl* ctl = a.ctl;
     unsigned long long* head = &ctl->tilectr[0].v;
@@ -834,10 +859,10 @@ __device__ __forceinline__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) 
     c.Fout = a.ring;
     c.cnt_out = tail;
     c.ring_cap = a.ring_cap;
-    seed_phase<POS, PK>(s, c, a);
+    seed_phase<POS, LAY>(s, c, a);
     block_flush(s, c);
     grid_sync(ctl);
-    async_loop<POS, PK>(s, c, a, head, tail, done);
+    async_loop<POS, LAY>(s, c, a, head, tail, done);
     grid_sync(ctl);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         *head = 0;
@@ -847,7 +872,7 @@ __device__ __forceinline__ void async_phase(Smem& s, Ctx& c, const PushArgs& a) 
     grid_sync(ctl);
 }
 
-template <bool PK>
+template <int LAY>
 __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid_constant__ PushArgs a) {
     __shared__ Smem s;
     Ctx c;
@@ -866,9 +891,9 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid
     grid_sync(a.ctl);
     const bool stamp = blockIdx.x == 0 && threadIdx.x == 0;
     const unsigned long long t0 = stamp ? globaltimer_ns() : 0;
-    if (a.phases & 1) async_phase<true, PK>(s, c, a);
+    if (a.phases & 1) async_phase<true, LAY>(s, c, a);
     const unsigned long long t1 = stamp ? globaltimer_ns() : 0;  // async_phase ends with a grid barrier
-    if (a.phases & 2) async_phase<false, PK>(s, c, a);
+    if (a.phases & 2) async_phase<false, LAY>(s, c, a);
     if (stamp) {  // phase durations, summed over launches (source waves)
         atomicAdd(&a.ctl->st.ns_push[0], t1 - t0);
         atomicAdd(&a.ctl->st.ns_push[1], globaltimer_ns() - t1);
@@ -885,34 +910,34 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_async(const __grid
     }
 }
 
-template <bool PK>
+template <int LAY>
 cudaError_t launch_async(const PushArgs& a, int num_sms, cudaStream_t st) {
     int bps = 0;
-    const cudaError_t e = blocks_per_sm((const void*)k_push_async<PK>, PT, PUSH_MIN_BLOCKS, &bps);
+    const cudaError_t e = blocks_per_sm((const void*)k_push_async<LAY>, PT, PUSH_MIN_BLOCKS, &bps);
     if (e != cudaSuccess) return e;
-    return coop_launch((const void*)k_push_async<PK>, num_sms * bps, a, st);
+    return coop_launch((const void*)k_push_async<LAY>, num_sms * bps, a, st);
 }
 
-template <int MODE, bool PK>
+template <int MODE, int LAY>
 cudaError_t launch_mode(const PushArgs& a, int num_sms, cudaStream_t st) {
     int bps = 0;
-    const cudaError_t e = blocks_per_sm((const void*)k_push<MODE, PK>, PT, PUSH_MIN_BLOCKS, &bps);
+    const cudaError_t e = blocks_per_sm((const void*)k_push<MODE, LAY>, PT, PUSH_MIN_BLOCKS, &bps);
     if (e != cudaSuccess) return e;
-    return coop_launch((const void*)k_push<MODE, PK>, num_sms * bps, a, st);
+    return coop_launch((const void*)k_push<MODE, LAY>, num_sms * bps, a, st);
 }
 
-template <bool PK>
+template <int LAY>
 cudaError_t launch_layout(int mode, const PushArgs& a, int num_sms, cudaStream_t st) {
 #if PPR_PUSH_OPT_ONLY
-    return mode == M_OPT ? launch_mode<M_OPT, PK>(a, num_sms, st) : cudaErrorInvalidValue;
+    return mode == M_OPT ? launch_mode<M_OPT, LAY>(a, num_sms, st) : cudaErrorInvalidValue;
 #endif
     switch (mode) {
-        case M_OPT: return launch_mode<M_OPT, PK>(a, num_sms, st);
-        case M_EAGER: return launch_mode<M_EAGER, PK>(a, num_sms, st);
-        case M_DUP: return launch_mode<M_DUP, PK>(a, num_sms, st);
-        case M_VAN: return launch_mode<M_VAN, PK>(a, num_sms, st);
-        case M_ASYNC: return launch_async<PK>(a, num_sms, st);
-        case M_SCAN: return launch_mode<M_SCAN, PK>(a, num_sms, st);
+        case M_OPT: return launch_mode<M_OPT, LAY>(a, num_sms, st);
+        case M_EAGER: return launch_mode<M_EAGER, LAY>(a, num_sms, st);
+        case M_DUP: return launch_mode<M_DUP, LAY>(a, num_sms, st);
+        case M_VAN: return launch_mode<M_VAN, LAY>(a, num_sms, st);
+        case M_ASYNC: return launch_async<LAY>(a, num_sms, st);
+        case M_SCAN: return launch_mode<M_SCAN, LAY>(a, num_sms, st);
         default: return cudaErrorInvalidValue;
     }
 }
@@ -926,8 +951,9 @@ cudaError_t launch_layout(int mode, const PushArgs& a, int num_sms, cudaStream_t
 #endif
 cudaError_t PPR_PUSH_ENTRY(int mode, const PushArgs& a, int num_sms, cudaStream_t st) {
     if (mode == 6 /* PPR_MODE_SHARED */) return a.g.rec ? cudaErrorInvalidValue : launch_push_ms(a, num_sms, st);
-    return a.g.rec ? launch_layout<true>(mode, a, num_sms, st)
-                   : launch_layout<false>(mode, a, num_sms, st);
+    if (a.g.rec) return launch_layout<LAY_PACKED>(mode, a, num_sms, st);
+    return a.g.pool_wide ? launch_layout<LAY_WIDE>(mode, a, num_sms, st)
+                         : launch_layout<LAY_ARRAYS>(mode, a, num_sms, st);
 }
 
 }  // namespace ppr

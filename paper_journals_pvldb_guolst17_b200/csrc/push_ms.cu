@@ -53,6 +53,9 @@ constexpr int NW = PT / 32;
 #endif
 constexpr int MT = PPR_MS_MT;  // frontier entries per CTA tile (a multiple of 32)
 static_assert(MT % 32 == 0, "MT");
+#ifndef PPR_MS_DIV
+#define PPR_MS_DIV 0
+#endif
 #ifndef PPR_MS_QW
 #define PPR_MS_QW 256
 #endif
@@ -78,7 +81,7 @@ struct MsSmem {
 };
 
 struct MsCtx {
-    const uint32_t* pool;
+    const PoolEnt* pool;
     unsigned long long* Fout;
     unsigned long long* cnt_out;
     uint32_t qn;
@@ -152,7 +155,7 @@ __device__ __forceinline__ int owner_of(const uint32_t* scan, uint32_t e, int to
 
 // ---------------------------------------------------------------- one tile
 
-template <bool POS>
+template <bool POS, bool WIDE>
 __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, uint32_t SG,
                                         const unsigned long long* Fin, uint64_t C, uint64_t base,
                                         uint32_t T, int top) {
@@ -295,11 +298,22 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
         uint32_t v = 0, d = 1;
         if (ok) {
             j = owner_of(scan, e, top);
-            v = ld_pool(&c.pool[s.off[j] + (e - scan[j])], pol_stream);
-            d = ld_dout(&a.g.dout[v], pol_keep);
+            const uint64_t i = s.off[j] + (e - scan[j]);
+            if constexpr (WIDE) {  // d_out(v) travels with the in-list entry
+                const PoolEnt pe = ld_pool_ent(&c.pool[i], pol_stream);
+                v = pe_v(pe);
+                d = pe_d(pe);
+            } else {
+                v = ld_u32_nc_pol(reinterpret_cast<const uint32_t*>(c.pool) + i, pol_stream);
+                d = ld_u32_nc_pol(&a.g.dout[v], pol_keep);
+            }
             mark(a.bitmap, (unsigned long long)v * SG + s.grp[j]);
         }
+#if PPR_MS_DIV  // experiment: every lane divides (as the oracle), no shared reciprocal
+        const double rd = (double)d;
+#else
         const double rd = __drcp_rn((double)d);
+#endif
         const uint32_t nk = E - cb * 32 < 32 ? E - cb * 32 : 32;
         for (uint32_t k = 0; k < nk; k++) {
             const uint32_t vk = __shfl_sync(0xffffffffu, v, k);
@@ -307,7 +321,11 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
             const double rk = __shfl_sync(0xffffffffu, rd, k);
             const double wl = s.w[jk][L];
             if (wl != 0.0)
+#if PPR_MS_DIV
+                red_add_pol(a.g.R + (size_t)vk * S + s.grp[jk] * 32 + L, __ddiv_rn(wl, rk), pol_keep);
+#else
                 red_add_pol(a.g.R + (size_t)vk * S + s.grp[jk] * 32 + L, __dmul_rn(wl, rk), pol_keep);
+#endif
         }
     }
     __syncthreads();  // smem of this tile is reused by the next
@@ -315,7 +333,7 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
 }
 
 // every CTA takes tiles of T entries (first statically, the rest by claims)
-template <bool POS>
+template <bool POS, bool WIDE>
 __device__ __forceinline__ void ms_round(MsSmem& s, MsCtx& c, const PushArgs& a, uint32_t SG,
                                          const unsigned long long* Fin, uint64_t C,
                                          unsigned long long* tc) {
@@ -333,7 +351,7 @@ __device__ __forceinline__ void ms_round(MsSmem& s, MsCtx& c, const PushArgs& a,
         // overlaps the tile (thread 0 first needs the result after it)
         unsigned long long claim = 0;
         if (PPR_MS_CLAIM_AHEAD && dyn && threadIdx.x == 0) claim = atomicAdd(tc, 1ull);
-        ms_tile<POS>(s, c, a, SG, Fin, C, t * T, T, top);  // ends with a CTA barrier
+        ms_tile<POS, WIDE>(s, c, a, SG, Fin, C, t * T, T, top);  // ends with a CTA barrier
         if (!dyn) break;
         if (!PPR_MS_CLAIM_AHEAD && threadIdx.x == 0) claim = atomicAdd(tc, 1ull);
         if (threadIdx.x == 0) s.next = claim + gridDim.x;
@@ -396,7 +414,7 @@ __device__ __forceinline__ void ms_seed(const PushArgs& a, uint32_t SG) {
     }
 }
 
-template <bool POS>
+template <bool POS, bool WIDE>
 __device__ __forceinline__ void ms_phase(MsSmem& s, MsCtx& c, const PushArgs& a, uint32_t SG,
                                          unsigned& it) {
     DevCtl* ctl = a.ctl;
@@ -426,7 +444,7 @@ __device__ __forceinline__ void ms_phase(MsSmem& s, MsCtx& c, const PushArgs& a,
         const unsigned long long* Fin = a.F[it & 1];
         c.Fout = a.F[(it + 1) & 1];
         c.cnt_out = &ctl->fcount[(it + 1) % 3].v;
-        ms_round<POS>(s, c, a, SG, Fin, C, &ctl->tilectr[it % 3].v);
+        ms_round<POS, WIDE>(s, c, a, SG, Fin, C, &ctl->tilectr[it % 3].v);
         grid_sync(ctl);  // every reduction and mark of the round has landed
         ms_scan(s, c, a, SG);
         block_flush(s, c);
@@ -442,6 +460,7 @@ __device__ __forceinline__ void ms_phase(MsSmem& s, MsCtx& c, const PushArgs& a,
     grid_sync(ctl);
 }
 
+template <bool WIDE>  // PoolEnt in-list entries carrying d_out (ppr_internal.cuh), else u32 ids
 __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_constant__ PushArgs a) {
     __shared__ MsSmem s;
     MsCtx c;
@@ -460,9 +479,9 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_co
     const bool stamp = blockIdx.x == 0 && threadIdx.x == 0;
     const unsigned long long t0 = stamp ? globaltimer_ns() : 0;
     unsigned it = 0;
-    if (a.phases & 1) ms_phase<true>(s, c, a, SG, it);
+    if (a.phases & 1) ms_phase<true, WIDE>(s, c, a, SG, it);
     const unsigned long long t1 = stamp ? globaltimer_ns() : 0;  // ms_phase ends with a grid barrier
-    if (a.phases & 2) ms_phase<false>(s, c, a, SG, it);
+    if (a.phases & 2) ms_phase<false, WIDE>(s, c, a, SG, it);
     if (stamp) {  // phase durations, summed over launches (source waves)
         atomicAdd(&a.ctl->st.ns_push[0], t1 - t0);
         atomicAdd(&a.ctl->st.ns_push[1], globaltimer_ns() - t1);
@@ -487,7 +506,8 @@ __global__ void __launch_bounds__(PT, PUSH_MIN_BLOCKS) k_push_ms(const __grid_co
 
 cudaError_t launch_push_ms(const PushArgs& a, int num_sms, cudaStream_t st) {
     int bps = 0;
-    const cudaError_t e = blocks_per_sm((const void*)k_push_ms, PT, PUSH_MIN_BLOCKS, &bps);
+    const void* fn = a.g.pool_wide ? (const void*)k_push_ms<true> : (const void*)k_push_ms<false>;
+    const cudaError_t e = blocks_per_sm(fn, PT, PUSH_MIN_BLOCKS, &bps);
     if (e != cudaSuccess) return e;
     PushArgs copy = a;
     void* args[] = {&copy};
@@ -511,7 +531,7 @@ cudaError_t launch_push_ms(const PushArgs& a, int num_sms, cudaStream_t st) {
     }
     cfg.attrs = at;
     cfg.numAttrs = na;
-    return cudaLaunchKernelExC(&cfg, (const void*)k_push_ms, args);
+    return cudaLaunchKernelExC(&cfg, fn, args);
 }
 
 }  // namespace ppr

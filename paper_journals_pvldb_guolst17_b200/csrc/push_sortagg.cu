@@ -101,7 +101,7 @@ __global__ void __launch_bounds__(SA_T) k_sa_self(const PushArgs a, const unsign
 }
 
 // one warp per frontier entry: its pairs at off[i] .. off[i] + |N_in(u)|
-__global__ void __launch_bounds__(SA_T) k_sa_gen(const PushArgs a, const uint32_t* pool,
+__global__ void __launch_bounds__(SA_T) k_sa_gen(const PushArgs a, const PoolEnt* pool,
                                                  const unsigned long long* F, uint64_t C,
                                                  const unsigned long long* off, const double* W,
                                                  uint64_t* keys, uint32_t* vals, double* inc) {
@@ -116,11 +116,12 @@ __global__ void __launch_bounds__(SA_T) k_sa_gen(const PushArgs a, const uint32_
         const double cw = __dmul_rn(c1, W[i]);  // (1 - a) * w_u, as the oracle's loop
         const unsigned long long o = off[i];
         for (uint32_t j = lane; j < sl.len; j += 32) {
-            const uint32_t x = pool[sl.off + j];
+            const uint32_t x = pool_id(a.g, pool, sl.off + j);
+            const uint32_t dx = a.g.pool_wide ? pe_d(pool[sl.off + j]) : a.g.dout[x];
             const uint64_t p = o + j;
             keys[p] = (uint64_t)x * S + sidx;
             vals[p] = (uint32_t)p;
-            inc[p] = __ddiv_rn(cw, (double)a.g.dout[x]);
+            inc[p] = __ddiv_rn(cw, (double)dx);
         }
     }
 }
@@ -233,7 +234,7 @@ template <bool POS>
 cudaError_t sa_phase(SortAgg* s, const PushArgs& a, uint64_t nv, cudaStream_t st,
                      SortAggStats* out, uint32_t* launches) {
     const uint64_t Sn = (uint64_t)a.g.S * a.g.n;
-    const uint32_t* pool = a.g.pool[out->active_pool];
+    const PoolEnt* pool = a.g.pool[out->active_pool];
     int shifts[8];
     const int bits = ceil_log2_u64(Sn);
     int np = 0;

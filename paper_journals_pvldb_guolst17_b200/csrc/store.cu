@@ -189,7 +189,7 @@ __global__ void k_store_validate(const __grid_constant__ DevGraph g, const uint6
     __syncthreads();
     const unsigned lane = threadIdx.x & 31u;
     const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
-    const uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->st.active_pool];
+    const PoolEnt* pool = g.pool[*(volatile unsigned*)&ctl->st.active_pool];
     const uint64_t warp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     if (force_rebuild && blockIdx.x == 0 && threadIdx.x == 0) ctl->st.rebuild = 1;
@@ -212,7 +212,7 @@ __global__ void k_store_validate(const __grid_constant__ DevGraph g, const uint6
             const uint32_t pb = p0 + lane * VQ;  // this lane's block of VQ positions
             uint32_t x[VQ];
 #pragma unroll
-            for (int q = 0; q < VQ; q++) x[q] = pb + q < sl.len ? pool[sl.off + pb + q] : 0u;
+            for (int q = 0; q < VQ; q++) x[q] = pb + q < sl.len ? pool_id(g, pool, sl.off + pb + q) : 0u;
             uint32_t cl = 0;  // claimed positions of the block (bit q)
 #pragma unroll
             for (int q = 0; q < VQ; q++) {
@@ -254,7 +254,7 @@ __device__ __forceinline__ void apply_segments(const DevGraph& g, const uint64_t
                                                uint64_t nwarps) {
     const unsigned lane = threadIdx.x & 31u;
     const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
-    uint32_t* pool = g.pool[*(volatile unsigned*)&ctl->st.active_pool];
+    PoolEnt* pool = g.pool[*(volatile unsigned*)&ctl->st.active_pool];
     for (uint64_t w = warp; w < nseg; w += nwarps) {
         const uint64_t i0 = b.vheads[w];
         const uint32_t v = (uint32_t)(kv[i0] >> 32);
@@ -271,7 +271,7 @@ __device__ __forceinline__ void apply_segments(const DevGraph& g, const uint64_t
             const unsigned m = __ballot_sync(0xffffffffu, filler);
             if (filler) {
                 const uint32_t hole = dp[filled + __popc(m & ((1u << lane) - 1u))];
-                pool[sl.off + hole] = pool[sl.off + t];
+                pool_copy(g, pool, sl.off + hole, pool, sl.off + t);
             }
             filled += __popc(m);
         }
@@ -290,9 +290,12 @@ __device__ __forceinline__ void apply_segments(const DevGraph& g, const uint64_t
             }
             uint32_t tot;
             const uint32_t ex = warp_excl_scan_u32(c, tot);
-            for (uint32_t k = 0; k < c; k++) pool[sl.off + pos + ex + k] = x;
+            // d_out(x) is filled in by the degree refresh after the restore (k_rebuild)
+            for (uint32_t k = 0; k < c; k++) pool_put(g, pool, sl.off + pos + ex + k, x, 0);
             pos += tot;
         }
+        // slots vacated when more copies were deleted than inserted become empty
+        for (uint32_t t = keep + I + lane; t < sl.len; t += 32) pool_clear(g, pool, sl.off + t);
         if (lane == 0) *lenp<PK>(g, v) = keep + I;
     }
 }
@@ -332,9 +335,9 @@ __device__ __forceinline__ uint32_t cap_for(uint32_t len, double slack, uint32_t
 
 // warp-wide stable copy of slab v into dst[no ..] without its claimed
 // deletions, followed by its net insertions; returns the new length
-__device__ uint32_t copy_merged_warp(const uint32_t* src, uint32_t* dst, const Slab sl,
-                                     unsigned long long no, const uint64_t* kv, const BatchBufs& b,
-                                     uint32_t sg) {
+__device__ uint32_t copy_merged_warp(const DevGraph& g, const PoolEnt* src, PoolEnt* dst, const Slab sl,
+                                     unsigned long long no, uint32_t cap, const uint64_t* kv,
+                                     const BatchBufs& b, uint32_t sg) {
     const unsigned lane = threadIdx.x & 31u;
     const uint32_t D = sg != NONE ? b.seg_D[sg] : 0u;
     const uint32_t* dp = sg != NONE ? b.delpos + sg : nullptr;
@@ -343,7 +346,7 @@ __device__ uint32_t copy_merged_warp(const uint32_t* src, uint32_t* dst, const S
         const uint32_t p = p0 + lane;
         const bool keep = p < sl.len && !(D && contains_u32(dp, D, p));
         const unsigned m = __ballot_sync(0xffffffffu, keep);
-        if (keep) dst[no + pos + __popc(m & ((1u << lane) - 1u))] = src[sl.off + p];
+        if (keep) pool_copy(g, dst, no + pos + __popc(m & ((1u << lane) - 1u)), src, sl.off + p);
         pos += __popc(m);
     }
     if (sg != NONE) {
@@ -360,15 +363,16 @@ __device__ uint32_t copy_merged_warp(const uint32_t* src, uint32_t* dst, const S
             }
             uint32_t tot;
             const uint32_t ex = warp_excl_scan_u32(c, tot);
-            for (uint32_t k = 0; k < c; k++) dst[no + pos + ex + k] = x;
+            for (uint32_t k = 0; k < c; k++) pool_put(g, dst, no + pos + ex + k, x, 0);  // degree: refresh
             pos += tot;
         }
     }
+    for (uint32_t t = pos + lane; t < cap; t += 32) pool_clear(g, dst, no + t);  // the slab's slack
     return pos;
 }
 
 template <bool PK>
-__device__ __forceinline__ void rebuild_body(const DevGraph& g, const uint64_t* __restrict__ kv,
+__device__ __forceinline__ unsigned long long rebuild_body(const DevGraph& g, const uint64_t* __restrict__ kv,
                                              const BatchBufs& b, const VertexBufs& vb, double slack,
                                              uint32_t min_cap, uint64_t cap0, uint64_t cap1,
                                              DevCtl* ctl) {
@@ -378,8 +382,8 @@ __device__ __forceinline__ void rebuild_body(const DevGraph& g, const uint64_t* 
     // the spare pool's capacity, read with the device-side active flag (a replayed
     // batch graph must not bake in the pool that was spare when it was captured)
     const uint64_t alt_cap = act ? cap0 : cap1;
-    const uint32_t* src = act ? g.pool[1] : g.pool[0];
-    uint32_t* dst = act ? g.pool[0] : g.pool[1];
+    const PoolEnt* src = act ? g.pool[1] : g.pool[0];
+    PoolEnt* dst = act ? g.pool[0] : g.pool[1];
     const unsigned lane = threadIdx.x & 31u;
     // contiguous vertex range of this CTA
     const uint64_t chunk = ((uint64_t)g.n + gridDim.x - 1) / gridDim.x;
@@ -413,7 +417,7 @@ __device__ __forceinline__ void rebuild_body(const DevGraph& g, const uint64_t* 
     if (blockIdx.x == 0 && threadIdx.x == 0) ctl->st.pool_top = total;
     if (total > alt_cap) {  // cannot happen: the host sizes the other pool (uniform exit)
         if (blockIdx.x == 0 && threadIdx.x == 0) atomicCAS(&ctl->st.err, KERR_OK, KERR_OVERFLOW);
-        return;
+        return 0;
     }
     // phase 3: offsets and the copy of short untouched slabs (thread per vertex);
     // long or changed slabs go to the warp-wide list
@@ -429,7 +433,8 @@ __device__ __forceinline__ void rebuild_body(const DevGraph& g, const uint64_t* 
             const Slab sl = get_slab<PK>(g, v);
             big = vb.vseg[v] != NONE || sl.len > 16;
             if (!big) {
-                for (uint32_t j = 0; j < sl.len; j++) dst[no + j] = src[sl.off + j];
+                for (uint32_t j = 0; j < sl.len; j++) pool_copy(g, dst, no + j, src, sl.off + j);
+                for (uint32_t j = sl.len; j < nc; j++) pool_clear(g, dst, no + j);
                 Slab ns;
                 ns.off = no;
                 ns.len = sl.len;
@@ -455,7 +460,7 @@ __device__ __forceinline__ void rebuild_body(const DevGraph& g, const uint64_t* 
         const uint32_t v = __ldcg(&vb.big[w]);
         const Slab sl = get_slab<PK>(g, v);
         const unsigned long long no = __ldcg(&vb.newoff[v]);
-        const uint32_t len = copy_merged_warp(src, dst, sl, no, kv, b, vb.vseg[v]);
+        const uint32_t len = copy_merged_warp(g, src, dst, sl, no, __ldcg(&vb.newcap[v]), kv, b, vb.vseg[v]);
         if (lane == 0) {
             Slab ns;
             ns.off = no;
@@ -466,24 +471,63 @@ __device__ __forceinline__ void rebuild_body(const DevGraph& g, const uint64_t* 
     }
     grid_sync(ctl);
     if (blockIdx.x == 0 && threadIdx.x == 0) ctl->st.active_pool = act ^ 1u;
+    return total;
 }
 
-// The rebuild (only if a slab would overflow; the decision is uniform: it was
-// made by the validation before this launch) and, with `cleanup`, the reset
-// of the batch's v -> segment map (k_seg_cleanup folded in: one launch fewer)
+// The end of a batch's store pipeline, one cooperative launch:
+//  * the rebuild (only if a slab would overflow; the decision is uniform: it was
+//    made by the validation before this launch);
+//  * with `finish`: the reset of the batch's v -> segment map, and the degree
+//    refresh -- every entry of the active pool whose cached d_out (PoolEnt) no
+//    longer matches d_out after this batch's restore is rewritten, a coalesced
+//    stream over the pool's [0, extent) with one d_out gather per entry.
 template <bool PK>
 __global__ void __launch_bounds__(RB_THREADS) k_rebuild(const __grid_constant__ DevGraph g,
                                                         const uint64_t* __restrict__ kv, BatchBufs b,
                                                         VertexBufs vb, double slack, uint32_t min_cap,
                                                         uint64_t cap0, uint64_t cap1, DevCtl* ctl,
-                                                        int cleanup) {
-    if (*(volatile int*)&ctl->st.err == KERR_OK && *(volatile int*)&ctl->st.rebuild)
-        rebuild_body<PK>(g, kv, b, vb, slack, min_cap, cap0, cap1, ctl);
-    if (cleanup) {
-        const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
-        for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nseg;
-             w += (uint64_t)gridDim.x * blockDim.x)
-            vb.vseg[kv[b.vheads[w]] >> 32] = NONE;
+                                                        int finish) {
+    const bool ok = *(volatile int*)&ctl->st.err == KERR_OK;
+    unsigned act = *(volatile unsigned*)&ctl->st.active_pool;  // read before any flip
+    unsigned long long ext = *(volatile unsigned long long*)&ctl->st.pool_extent;
+    if (ok && *(volatile int*)&ctl->st.rebuild) {
+        const unsigned long long e = rebuild_body<PK>(g, kv, b, vb, slack, min_cap, cap0, cap1, ctl);
+        if (e) {
+            act ^= 1u;
+            ext = e;
+            if (blockIdx.x == 0 && threadIdx.x == 0) ctl->st.pool_extent = e;
+        }
+    }
+    if (!finish) return;
+    const uint64_t tid = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    const uint64_t nth = (uint64_t)gridDim.x * blockDim.x;
+    const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
+    for (uint64_t w = tid; w < nseg; w += nth) vb.vseg[kv[b.vheads[w]] >> 32] = NONE;
+    if (!ok || !g.pool_wide || !*(volatile unsigned*)&ctl->st.n_touched) return;  // nothing cached changed
+    // stream the active pool; gather d_out for every entry (8 gathers in flight per
+    // thread) and rewrite the stale ones.  (Testing a bitmap of the batch's touched
+    // vertices first was slower: its gather costs as much as the hub-concentrated
+    // d_out gather -- Twitter shape 19.4 vs 9.9 ms per batch.)
+    PoolEnt* pool = g.pool[act];
+    constexpr int RQ = 8;
+    for (uint64_t p0 = tid; p0 < ext; p0 += nth * RQ) {
+        PoolEnt e[RQ];
+        uint32_t d[RQ];
+#pragma unroll
+        for (int q = 0; q < RQ; q++) {
+            const uint64_t p = p0 + (uint64_t)q * nth;
+            e[q] = p < ext ? __ldcs(&pool[p]) : POOL_EMPTY;
+        }
+#pragma unroll
+        for (int q = 0; q < RQ; q++) {
+            const uint32_t v = pe_v(e[q]);
+            d[q] = v != 0xFFFFFFFFu ? *doutp<PK>(g, v) : 0u;  // empty slots are skipped
+        }
+#pragma unroll
+        for (int q = 0; q < RQ; q++) {
+            const uint32_t v = pe_v(e[q]);
+            if (v != 0xFFFFFFFFu && pe_d(e[q]) != d[q]) pool[p0 + (uint64_t)q * nth] = pe_make(v, d[q]);
+        }
     }
 }
 
@@ -655,15 +699,15 @@ __global__ void k_set_slabs(const __grid_constant__ DevGraph g, const unsigned l
 template <bool PK>
 __global__ void k_build_fill(const uint32_t* __restrict__ src, const uint32_t* __restrict__ dst,
                              uint64_t m, int undirected, const __grid_constant__ DevGraph g) {
-    uint32_t* pool = g.pool[0];
+    PoolEnt* pool = g.pool[0];  // d_out is final here (k_build_count)
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < m;
          i += (uint64_t)gridDim.x * blockDim.x) {
         const uint32_t u = src[i], v = dst[i];
         uint32_t p = atomicAdd(lenp<PK>(g, v), 1u);
-        pool[get_slab<PK>(g, v).off + p] = u;
+        pool_put(g, pool, get_slab<PK>(g, v).off + p, u, *doutp<PK>(g, u));
         if (undirected && u != v) {
             p = atomicAdd(lenp<PK>(g, u), 1u);
-            pool[get_slab<PK>(g, u).off + p] = v;
+            pool_put(g, pool, get_slab<PK>(g, u).off + p, v, *doutp<PK>(g, v));
         }
     }
 }
@@ -685,13 +729,13 @@ __global__ void k_len_to_u32(const __grid_constant__ DevGraph g, uint32_t* __res
 template <bool PK>
 __global__ void k_export(const __grid_constant__ DevGraph g, int active, const unsigned long long* __restrict__ off,
                          uint64_t* __restrict__ keys, const uint32_t* __restrict__ inv) {
-    const uint32_t* pool = g.pool[active];
+    const PoolEnt* pool = g.pool[active];
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < g.n;
          v += (uint64_t)gridDim.x * blockDim.x) {
         const Slab sl = get_slab<PK>(g, v);
         const uint64_t vo = inv ? inv[v] : v;  // external id
         for (uint32_t j = 0; j < sl.len; j++) {
-            const uint32_t x = pool[sl.off + j];
+            const uint32_t x = pool_id(g, pool, sl.off + j);
             keys[off[v] + j] = (vo << 32) | (inv ? inv[x] : x);
         }
     }
@@ -829,7 +873,7 @@ void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const
 
 cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                                  const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
-                                 cudaStream_t st, uint32_t* launches, bool cleanup) {
+                                 cudaStream_t st, uint32_t* launches, bool finish) {
     (void)N;
     const void* fn = g.rec ? (const void*)k_rebuild<true> : (const void*)k_rebuild<false>;
     int per_sm = 0, sms = 0, dev = 0;
@@ -846,7 +890,7 @@ cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t
     uint32_t min_cap = sp.min_cap;
     uint64_t cap0 = sp.cap0, cap1 = sp.cap1;
     DevCtl* c = ctl;
-    int cl = cleanup ? 1 : 0;
+    int cl = finish ? 1 : 0;
     void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &cap0, &cap1, &c, &cl};
     e = cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(RB_THREADS), args, 0, st);
     ++*launches;

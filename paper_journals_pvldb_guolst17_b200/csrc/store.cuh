@@ -65,10 +65,11 @@ void launch_store_validate(const DevGraph& g, const uint64_t* kv, uint64_t N, co
 void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                         DevCtl* ctl, cudaStream_t st, uint32_t* launches);
 // a1: sort/merge rebuild into the other pool (skipped unless DevCtl::rebuild)
-// (cleanup: also reset the v -> segment map, i.e. launch_seg_cleanup folded in)
+// (finish: also reset the v -> segment map and refresh the degrees cached in the
+// pool entries after the restore -- the last launch of every batch's store pipeline)
 cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                                  const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
-                                 cudaStream_t st, uint32_t* launches, bool cleanup = false);
+                                 cudaStream_t st, uint32_t* launches, bool finish);
 void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, const VertexBufs& vb,
                         DevCtl* ctl, cudaStream_t st, uint32_t* launches);
 

@@ -38,7 +38,7 @@ class Graph(ctypes.Structure):
 class Opts(ctypes.Structure):
     _fields_ = [("device", ctypes.c_int), ("cuda_stream", ctypes.c_void_p), ("mode", ctypes.c_int),
                 ("slack", ctypes.c_double), ("min_cap", ctypes.c_uint32), ("relabel", ctypes.c_int),
-                ("layout", ctypes.c_int), ("l2_persist", ctypes.c_int)]
+                ("layout", ctypes.c_int), ("l2_persist", ctypes.c_int), ("pool_degrees", ctypes.c_int)]
 
 
 class BatchStats(ctypes.Structure):
@@ -138,7 +138,7 @@ class Ppr:
 
     def __init__(self, n, src, dst, sources, alpha=0.15, eps=1e-9, mode="opt", device=0,
                  stream=None, undirected=False, slack=0.25, min_cap=4, relabel=-1,
-                 layout=LAYOUT_ARRAYS, l2_persist=-1):
+                 layout=LAYOUT_ARRAYS, l2_persist=-1, pool_degrees=-1):
         lib = load()
         s, sp = _host_u32(src)
         d, dp = _host_u32(dst)
@@ -148,7 +148,7 @@ class Ppr:
                   dst=ctypes.cast(dp, ctypes.POINTER(ctypes.c_uint32)), undirected=int(undirected))
         o = Opts(device=int(device), cuda_stream=stream, mode=MODES.get(mode, mode),
                  slack=float(slack), min_cap=int(min_cap), relabel=int(relabel),
-                 layout=int(layout), l2_persist=int(l2_persist))
+                 layout=int(layout), l2_persist=int(l2_persist), pool_degrees=int(pool_degrees))
         h = ctypes.c_void_p()
         st = BatchStats()
         rc = lib.ppr_create(ctypes.byref(g), ctypes.cast(sop, ctypes.POINTER(ctypes.c_uint32)),

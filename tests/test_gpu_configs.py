@@ -106,14 +106,16 @@ def test_orkut_big_deletion_heavy_batch(orkut_small, rebuild):
 def test_twitter_reduced_launch_configuration():
     """configs[3] protocol at n = 2e6: the window holds all but the last slides'
     insertions (resident), 12 arcs per vertex (dense), hub-band source;
-    relabelling forced on and the persisting L2 window off, as the library
-    chooses for the 41.6M-vertex shape (R + d_out = 500 MB)."""
+    relabelling forced on, the persisting L2 window off and degree-carrying
+    pool entries on, as the library chooses for the 41.6M-vertex shape
+    (R + d_out = 500 MB)."""
     st, cfg = W.make_stream("twitter", n=2_000_000, m=24_000_000, ins=10_000, dele=10_000,
                             slides=3)
     eps = 1e-9
     g0s, g0d = st.window()
     (s,) = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 1)
-    h = ppr.Ppr(cfg["n"], g0s, g0d, [s], alpha=ALPHA, eps=eps, relabel=1, l2_persist=0)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, [s], alpha=ALPHA, eps=eps, relabel=1, l2_persist=0,
+                pool_degrees=1)
     o = oracle.Oracle(cfg["n"], g0s, g0d, [s], ALPHA, eps)
     o.push(oracle.SEQ)
     check_batch_state(h, o, 0, int(s), eps, "twitter static")

@@ -97,7 +97,7 @@ _check_batch_state = check_batch_state
 
 
 def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, relabel=-1, options=None,
-                layout=ppr.LAYOUT_ARRAYS, **over):
+                layout=ppr.LAYOUT_ARRAYS, pool_degrees=-1, **over):
     """Streams `slides` batches through a handle and the oracle, checking the
     per-batch gates.  `options`: {ppr.OPT_*: value} set through ppr_set_option
     after create (schedule / kernel selection for the batches)."""
@@ -106,7 +106,7 @@ def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, relabel=
     g0s, g0d = st.window()
     srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], sources)
     h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=eps, mode=mode,
-                undirected=False, relabel=relabel, layout=layout)
+                undirected=False, relabel=relabel, layout=layout, pool_degrees=pool_degrees)
     for k, v in (options or {}).items():
         h.set_option(k, v)
     o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, eps)
@@ -130,6 +130,22 @@ def _run_stream(name, mode, slides, eps=None, sources=1, check_every=1, relabel=
 @pytest.mark.parametrize("mode", MODES)
 def test_tiny_config_all_modes_track_oracle(mode):
     _run_stream("tiny", mode, slides=12)
+
+
+@pytest.mark.parametrize("mode", MODES)
+def test_wide_pool_entries_track_oracle(mode):
+    # ppr_opts.pool_degrees = 1: in-list entries carry (d_out(u), u), refreshed after
+    # every restore (the format the library picks for DRAM-resident residuals)
+    _run_stream("tiny", mode, slides=8, pool_degrees=1, sources=3 if mode == "shared" else 1)
+
+
+@pytest.mark.parametrize("rebuild", [0, 1])
+def test_wide_pool_entries_rebuild_and_relabel(rebuild):
+    _run_stream("tiny", "opt", slides=6, pool_degrees=1, relabel=1,
+                options={ppr.OPT_FORCE_REBUILD: rebuild, ppr.OPT_RING_ALL: 1})
+    with pytest.raises(ppr.PprError) as ex:  # the packed records keep u32 in-list entries
+        _run_stream("tiny", "opt", slides=1, pool_degrees=1, layout=ppr.LAYOUT_PACKED)
+    assert ex.value.code == ppr.PPR_EINVAL
 
 
 @pytest.mark.parametrize("tail,ring_all", [(0, 0), (16384, 0), (16384, 1), (64, 0)])

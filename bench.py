@@ -93,6 +93,10 @@ def parse():
                    help="process-group backend (gloo: the multi-rank path on one GPU)")
     p.add_argument("--relabel", type=int, default=-1,
                    help="1: degree-ordered internal ids, 0: external ids, -1: by size (default)")
+    p.add_argument("--set", action="append", default=[], metavar="KEY=VALUE",
+                   help="ppr_set_option(KEY, VALUE) after create (PPR_OPT_* numbers; schedule A/B runs)")
+    p.add_argument("--pool-degrees", type=int, default=-1,
+                   help="1: in-list entries carry d_out, 0: u32 entries, -1: by size (default)")
     a = p.parse_args()
     if a.workload is None:
         a.workload = "lj" if a.gpus == 1 else "ms-lj"
@@ -452,9 +456,12 @@ def measure(args, cx, workload, S_total, with_e2e, with_cpu):
     t0 = time.perf_counter()
     h = ppr.Ppr(cfg["n"], win_np[0], win_np[1], my_srcs, alpha=0.15, eps=eps, mode=mode,
                 device=cx.local, stream=cx.stream.cuda_stream, undirected=und,
-                relabel=args.relabel)
+                relabel=args.relabel, pool_degrees=args.pool_degrees)
     if wave:
         h.set_option(ppr.OPT_WAVE, wave)
+    for kv in args.set:
+        k, v = kv.split("=")
+        h.set_option(int(k), int(v))
     torch.cuda.synchronize()
     t_create = time.perf_counter() - t0
     create_stats = h.create_stats

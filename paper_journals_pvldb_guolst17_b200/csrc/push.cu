@@ -55,6 +55,15 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_PUSH_U
 #define PPR_PUSH_U 2
 #endif
+#ifndef PPR_PUSH_TMAX
+#define PPR_PUSH_TMAX PT
+#endif
+#ifndef PPR_PUSH_PREF
+#define PPR_PUSH_PREF 0
+#endif
+#ifndef PPR_PUSH_PIPE
+#define PPR_PUSH_PIPE 1
+#endif
 #ifndef PPR_PUSH_OPT_ONLY
 #define PPR_PUSH_OPT_ONLY 0
 #endif
@@ -82,8 +91,21 @@ struct TileArrays {
     unsigned long long off[PT];           // slab offset of each entry
     double w[PT];                         // (1-a) * r of each entry
 };
+// PPR_PUSH_LEAN (default 1): two tile buffers alternate between consecutive
+// tiles of a round and the next tile is claimed as a tile starts, so a tile
+// costs two CTA barriers (warp totals, prefix) instead of six; warps that
+// finish walking tile t go on to tile t+1's entry loads and exchange while
+// the last warps of tile t are still walking (the barrier after the warp
+// totals of t+1 is the first point that waits for them).
+#ifndef PPR_PUSH_LEAN
+#define PPR_PUSH_LEAN 1
+#endif
+constexpr int NBUF = PPR_PUSH_LEAN ? 2 : 1;
 struct Smem {
-    TileArrays t;                         // the CTA's current tile
+    TileArrays tb[NBUF];                  // the CTA's current tile (LEAN: alternating buffers)
+    uint32_t wtot[NBUF][NW];              // LEAN: per-warp in-degree totals of a tile
+    unsigned long long nxt[NBUF];         // LEAN: the tile claimed while this one runs
+    unsigned int chunkb[NBUF];            // LEAN: next 32-edge chunk of each buffer
     unsigned long long q[NW][QW];         // per-warp enqueue slices
     unsigned int wq[NW];                  // slice fill at the end-of-round flush
     unsigned long long gbase;
@@ -201,7 +223,9 @@ __device__ __forceinline__ int owner_of(const uint32_t* scan, uint32_t e, int to
 template <bool POS, int KIND, int LAY>
 __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
                                           unsigned long long ent, uint64_t idx, uint32_t T,
-                                          int top);
+                                          int top, int buf = 0, unsigned long long nxt = 0,
+                                          unsigned long long* pf = nullptr,
+                                          const unsigned long long* Fin = nullptr, uint64_t C = 0);
 
 // Processes the T entries Fin[base_idx .. base_idx+T) (thread i = entry i):
 // neighbour propagation of every pushed entry and, for K_OPT, the fused
@@ -209,11 +233,12 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
 template <bool POS, int KIND, int LAY>
 __device__ __forceinline__ void cta_tile(Smem& s, Ctx& c, const PushArgs& a,
                                          const unsigned long long* Fin, uint64_t C,
-                                         uint64_t base_idx, uint32_t T, int top) {
+                                         uint64_t base_idx, uint32_t T, int top, int buf = 0,
+                                         unsigned long long nxt = 0) {
     const uint64_t idx = base_idx + threadIdx.x;
     const bool valid = threadIdx.x < T && idx < C;
     const unsigned long long ent = valid ? __ldcg(&Fin[idx]) : 0ull;
-    tile_body<POS, KIND, LAY>(s, c, a, valid, ent, idx, T, top);
+    tile_body<POS, KIND, LAY>(s, c, a, valid, ent, idx, T, top, buf, nxt);
 }
 
 // in-list entry i of the active pool: v, and d_out(v) for the wide format
@@ -271,6 +296,73 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
                 }
             }
         }
+    } else if constexpr (PPR_PUSH_PIPE) {
+    // software-pipelined walk: the next claim's pool entries are loaded while
+    // this claim's atomics are in flight, so a warp step costs about one
+    // atomic round trip instead of pool load + d_out gather + atomic
+    uint32_t cb = 0;
+    if (L == 0) cb = atomicAdd(chunkp, (unsigned)U);
+    cb = __shfl_sync(0xffffffffu, cb, 0);
+    uint32_t v[U], dw[U];
+    int j[U];
+#pragma unroll
+    for (int k = 0; k < U; k++) {
+        const uint32_t e = (cb + k) * 32 + L;
+        j[k] = -1;
+        v[k] = 0;
+        dw[k] = 1;
+        if (e < E) {
+            j[k] = owner_of(t.scan, e, top);
+            load_entry<LAY>(c.pool, t.off[j[k]] + (e - t.scan[j[k]]), pol_stream, v[k], dw[k]);
+        }
+    }
+    while (cb * 32 < E) {
+        ensure_room(s, c, 32 * U);
+        uint32_t d[U];
+#pragma unroll
+        for (int k = 0; k < U; k++)
+            d[k] = (LAY == LAY_WIDE || j[k] < 0) ? dw[k]
+                   : ((LAY == LAY_PACKED) ? __ldcg(&a.g.rec[v[k]].dout) : ld_u32_nc_pol(&a.g.dout[v[k]], pol_keep));
+        double incr[U], pre[U];
+        unsigned long long ev[U];
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            if (j[k] >= 0) {
+                const uint32_t sj = t.sid[j[k]];
+                incr[k] = __ddiv_rn(t.w[j[k]], (double)d[k]);
+                pre[k] = atom_add_pol(Rp<(LAY == LAY_PACKED)>(a.g, sj, v[k]), incr[k], pol_keep);
+                ev[k] = ((unsigned long long)sj << 32) | v[k];
+            }
+        }
+        bool act[U];
+#pragma unroll
+        for (int k = 0; k < U; k++) act[k] = j[k] >= 0;
+        // next claim: entries in flight with the atomics above
+        if (L == 0) cb = atomicAdd(chunkp, (unsigned)U);
+        cb = __shfl_sync(0xffffffffu, cb, 0);
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            const uint32_t e = (cb + k) * 32 + L;
+            j[k] = -1;
+            if (e < E) {
+                j[k] = owner_of(t.scan, e, top);
+                load_entry<LAY>(c.pool, t.off[j[k]] + (e - t.scan[j[k]]), pol_stream, v[k], dw[k]);
+            }
+        }
+#pragma unroll
+        for (int k = 0; k < U; k++) {
+            bool enq = false;
+            if (act[k]) {
+                const double cur = __dadd_rn(pre[k], incr[k]);  // == the stored value (no FMA)
+                if (KIND == K_OPT || KIND == K_DUP)
+                    enq = crossed<POS>(pre[k], cur, eps);   // Alg 4 line 16
+                else
+                    enq = push_cond<POS>(cur, eps) &&
+                          test_and_set(a.bitmap, (size_t)(ev[k] >> 32) * n + (uint32_t)ev[k]);  // UniqueEnqueue
+            }
+            warp_enqueue(s, c, enq, ev[k]);
+        }
+    }
     } else {
     // warps claim U consecutive 32-edge chunks at a time from a shared counter,
     // so a warp whose atomics return late does not hold up the others
@@ -334,7 +426,9 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
 template <bool POS, int KIND, int LAY>
 __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bool valid,
                                           unsigned long long ent, uint64_t idx, uint32_t T,
-                                          int top) {
+                                          int top, int buf, unsigned long long nxt,
+                                          unsigned long long* pf, const unsigned long long* Fin,
+                                          uint64_t C) {
     const double eps = a.g.eps, alpha = a.g.alpha;
     const uint32_t sidx = (uint32_t)(ent >> 32), u = (uint32_t)ent;
     double* ru = Rp<(LAY == LAY_PACKED)>(a.g, sidx, u);
@@ -379,22 +473,61 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
     if (!push) len = 0;
     if (push && KIND != K_VAN && KIND != K_DUP && KIND != K_EAGER) c.pushes++;
     uint32_t E;
-    const uint32_t ex = block_exclusive_scan_u32<PT>(len, s.warp_tmp, &E);
-    s.t.scan[threadIdx.x] = threadIdx.x < T ? ex : 0xFFFFFFFFu;
-    if (threadIdx.x == 0) {
-        s.t.scan[PT] = 0xFFFFFFFFu;
-        s.chunk = 0;
+    TileArrays& t = s.tb[buf];
+    unsigned int* chunkp = &s.chunk;
+    if constexpr (PPR_PUSH_LEAN) {
+        // two barriers: warp-inclusive scans + per-warp totals, then every warp
+        // scans the NW totals itself and writes its part of the prefix
+        const unsigned L = lane(), wi = warp();
+        uint32_t inc = len;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const uint32_t y = __shfl_up_sync(0xffffffffu, inc, o);
+            if (L >= (unsigned)o) inc += y;
+        }
+        if (L == 31) s.wtot[buf][wi] = inc;
+        t.off[threadIdx.x] = off;
+        t.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
+        t.sid[threadIdx.x] = sidx;
+        if (threadIdx.x == 0) {
+            t.scan[PT] = 0xFFFFFFFFu;
+            s.chunkb[buf] = 0;
+            s.nxt[buf] = nxt;
+        }
+        __syncthreads();
+        if (pf) {  // PREF: the next tile's entry of this thread, in flight during the walk
+            const uint64_t j = s.nxt[buf] * T + threadIdx.x;
+            *pf = (threadIdx.x < T && j < C) ? __ldcg(&Fin[j]) : 0ull;
+        }
+        const uint32_t wt = L < (unsigned)NW ? s.wtot[buf][L] : 0u;
+        uint32_t wsc = wt;
+#pragma unroll
+        for (int o = 1; o < NW; o <<= 1) {
+            const uint32_t y = __shfl_up_sync(0xffffffffu, wsc, o);
+            if (L >= (unsigned)o) wsc += y;
+        }
+        const uint32_t wbase = __shfl_sync(0xffffffffu, wsc - wt, wi);
+        E = __shfl_sync(0xffffffffu, wsc, NW - 1);
+        t.scan[threadIdx.x] = threadIdx.x < T ? wbase + inc - len : 0xFFFFFFFFu;
+        chunkp = &s.chunkb[buf];
+    } else {
+        const uint32_t ex = block_exclusive_scan_u32<PT>(len, s.warp_tmp, &E);
+        t.scan[threadIdx.x] = threadIdx.x < T ? ex : 0xFFFFFFFFu;
+        if (threadIdx.x == 0) {
+            t.scan[PT] = 0xFFFFFFFFu;
+            s.chunk = 0;
+        }
+        t.off[threadIdx.x] = off;
+        t.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
+        t.sid[threadIdx.x] = sidx;
     }
-    s.t.off[threadIdx.x] = off;
-    s.t.w[threadIdx.x] = __dmul_rn(1.0 - alpha, r);
-    s.t.sid[threadIdx.x] = sidx;
     __syncthreads();
     if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_pro += globaltimer_ns() - c.t_mark;
     if (threadIdx.x == 0) {
         c.edges += E;
         if (c.trace_edges && E) atomicAdd(c.trace_edges, (unsigned long long)E);
     }
-    walk_edges<POS, KIND, LAY>(s, c, a, s.t, E, top, &s.chunk);
+    walk_edges<POS, KIND, LAY>(s, c, a, t, E, top, chunkp);
 }
 
 // Every CTA takes tiles of T entries: its first tile statically, the rest by
@@ -404,12 +537,33 @@ __device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a
                               uint64_t C, unsigned long long* tc) {
     uint64_t per = (C + gridDim.x - 1) / gridDim.x;
     uint32_t T = (uint32_t)((per + 31) / 32 * 32);
-    if (T > PT) T = PT;
+    if (T > PPR_PUSH_TMAX) T = PPR_PUSH_TMAX;
     if (T < 32) T = 32;
     int top = 1;
     while (top * 2 < (int)T) top <<= 1;
     const uint64_t ntiles = (C + T - 1) / T;
     uint64_t t = blockIdx.x;
+    if constexpr (PPR_PUSH_LEAN) {
+        // the claim of the next tile is issued as a tile starts and published
+        // with the tile's first barrier; buffers alternate (see Smem)
+        const bool claims = ntiles > gridDim.x;
+        int buf = 0;
+        unsigned long long pent = 0;
+        bool have = false;
+        while (t < ntiles) {
+            unsigned long long nxt = ~0ull;
+            if (claims && threadIdx.x == 0) nxt = atomicAdd(tc, 1ull) + gridDim.x;
+            const uint64_t idx = t * T + threadIdx.x;
+            const bool valid = threadIdx.x < T && idx < C;
+            const unsigned long long ent = have ? pent : (valid ? __ldcg(&Fin[idx]) : 0ull);
+            tile_body<POS, KIND, LAY>(s, c, a, valid, ent, idx, T, top, buf, nxt,
+                                      (PPR_PUSH_PREF && claims) ? &pent : nullptr, Fin, C);
+            have = PPR_PUSH_PREF && claims;
+            t = claims ? s.nxt[buf] : ntiles;
+            buf ^= 1;
+        }
+        __syncthreads();  // every warp is done with both buffers before the round's flush
+    } else {
     while (t < ntiles) {
         if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_mark = globaltimer_ns();
         cta_tile<POS, KIND, LAY>(s, c, a, Fin, C, t * T, T, top);
@@ -420,6 +574,7 @@ __device__ __forceinline__ void propagate_all(Smem& s, Ctx& c, const PushArgs& a
         t = s.next;
         __syncthreads();
         if (kTimeSplit && a.trace && threadIdx.x == 0) c.t_claim += globaltimer_ns() - c.t_mark2;
+    }
     }
 }
 

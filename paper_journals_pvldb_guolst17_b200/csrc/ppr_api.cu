@@ -80,7 +80,8 @@ struct ppr_ctx {
     size_t l2_win_bytes = 0;
     float l2_hit = 0.f;
     uint32_t* d_dout = nullptr;  // structure-of-arrays layout (S > 1)
-    Slab* d_slab = nullptr;
+    SlabRec* d_slab = nullptr;   // {off, len} of N_in(v) (ppr_internal.cuh)
+    uint32_t* d_cap = nullptr;   // slab capacities
     PoolEnt* d_pool[2] = {nullptr, nullptr};  // slab pools (entries: PoolEnt if pool_wide, else u32)
     bool pool_wide = false;                   // ppr_opts.pool_degrees (ppr_internal.cuh PoolEnt)
     double* d_P = nullptr;
@@ -215,6 +216,9 @@ void dfree(ppr_ctx* h, T*& p, uint64_t count) {
 }
 
 // PoolEnt-sized words backing a pool of `cap` entries (4 or 8 bytes each)
+// slab offsets are u32 (SlabRec), so a pool holds at most this many entries
+constexpr uint64_t kPoolMaxEntries = 0xFFFFFFFFull - 64;
+
 uint64_t pool_words(const ppr_ctx* h, uint64_t cap) { return h->pool_wide ? cap : (cap + 1) / 2; }
 
 DevGraph graph_of(const ppr_ctx* h) {
@@ -225,6 +229,7 @@ DevGraph graph_of(const ppr_ctx* h) {
     g.eps = h->eps;
     g.dout = h->d_dout;
     g.slab = h->d_slab;
+    g.cap = h->d_cap;
     g.pool[0] = h->d_pool[0];
     g.pool[1] = h->d_pool[1];
     g.pool_wide = h->pool_wide ? 1u : 0u;
@@ -303,12 +308,17 @@ ppr_status ensure_alt_pool(ppr_ctx* h, uint64_t new_arcs) {
         std::ceil((1.0 + h->slack) * (double)(h->m + new_arcs)) + (double)(h->min_cap + 1) * h->n + 1024;
     const uint64_t need = (uint64_t)need_d;
     if (h->pool_cap[alt] >= need) return PPR_OK;
+    if (need > kPoolMaxEntries) {
+        set_err(h, "a slab pool of %llu entries exceeds the 2^32 - 1 entries u32 slab offsets address",
+                (unsigned long long)need);
+        return PPR_ENOMEM;
+    }
     cudaError_t e = cudaStreamSynchronize(h->st);
     if (e != cudaSuccess) return cuda_fail(h, e, "ensure_alt_pool sync");
     dfree(h, h->d_pool[alt], pool_words(h, h->pool_cap[alt]));
     h->pool_cap[alt] = 0;
     h->buf_epoch++;
-    uint64_t cap = need + need / 4;
+    uint64_t cap = std::min<uint64_t>(need + need / 4, kPoolMaxEntries);
     if (dalloc(h, &h->d_pool[alt], pool_words(h, cap)) != cudaSuccess) {
         set_err(h, "out of device memory for the rebuild pool (%llu entries)",
                 (unsigned long long)cap);
@@ -445,6 +455,7 @@ void destroy_all(ppr_ctx* h) {
     }
     dfree(h, h->d_dout, h->n);
     dfree(h, h->d_slab, h->n);
+    dfree(h, h->d_cap, h->n);
     dfree(h, h->d_pool[0], pool_words(h, h->pool_cap[0]));
     dfree(h, h->d_pool[1], pool_words(h, h->pool_cap[1]));
     dfree(h, h->d_P, (uint64_t)h->S * h->n);
@@ -747,6 +758,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
     bool ok = packed ? dalloc(h, &h->d_rec, h->n) == cudaSuccess
                      : (dalloc(h, &h->d_hot, Sn + (h->n + 1) / 2 + 32) == cudaSuccess &&
                         dalloc(h, &h->d_slab, h->n) == cudaSuccess &&
+                        dalloc(h, &h->d_cap, h->n) == cudaSuccess &&
                         dalloc(h, &h->d_P, Sn) == cudaSuccess);
     if (ok && !packed) {
         h->d_R = h->d_hot;
@@ -813,7 +825,8 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         cudaMemsetAsync(h->d_rec, 0, sizeof(VRec) * h->n, st);
     } else {
         cudaMemsetAsync(h->d_dout, 0, sizeof(uint32_t) * h->n, st);
-        cudaMemsetAsync(h->d_slab, 0, sizeof(Slab) * h->n, st);
+        cudaMemsetAsync(h->d_slab, 0, sizeof(SlabRec) * h->n, st);
+        cudaMemsetAsync(h->d_cap, 0, sizeof(uint32_t) * h->n, st);
         cudaMemsetAsync(h->d_P, 0, sizeof(double) * Sn, st);
         cudaMemsetAsync(h->d_R, 0, sizeof(double) * Sn, st);
     }
@@ -882,7 +895,16 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
                             (double)(h->min_cap + 1) * h->n + 1024;
         uint64_t cap = (uint64_t)(need + need / 4);
         if (cap < total + 1024) cap = total + 1024;
+        if (cap > kPoolMaxEntries) cap = std::max<uint64_t>((uint64_t)need, total + 1024);
         h->pool_cap[0] = h->pool_cap[1] = cap;
+    }
+    if (h->pool_cap[0] > kPoolMaxEntries) {  // u32 slab offsets (SlabRec)
+        dfree(h, d_src, g->m);
+        dfree(h, d_dst, g->m);
+        set_err(h, "the graph needs a slab pool beyond 2^32 - 1 entries");
+        destroy_all(h);
+        delete h;
+        return PPR_ENOMEM;
     }
     if (dalloc(h, &h->d_pool[0], pool_words(h, h->pool_cap[0])) != cudaSuccess ||
         dalloc(h, &h->d_pool[1], pool_words(h, h->pool_cap[1])) != cudaSuccess) {

@@ -3,7 +3,7 @@
 //
 // HBM layout:
 //   dout   u32[n]                 d_out(v)                       (Table 1)
-//   slab   Slab[n] (16 B each)    {u64 off, u32 len, u32 cap} of N_in(v)
+//   slab   SlabRec[n] (8 B each) {u32 off, u32 len} of N_in(v); cap u32[n] (store only)
 //   pool   u32[pool_cap] x 2      slab storage; one active, one rebuild target
 //   P, R   f64[S][n]              estimate / residual per source (Table 1)
 //   F      u64[S*n] x 2           frontier entries (sidx << 32 | v), double-buffered
@@ -16,10 +16,20 @@
 
 namespace ppr {
 
-struct __align__(16) Slab {
+// Logical slab descriptor of N_in(v) (what the store code works with).
+struct Slab {
     unsigned long long off;  // first pool index of N_in(v)
     uint32_t len;            // |N_in(v)| (multiset)
     uint32_t cap;            // reserved entries
+};
+// Stored form (array layout): the push reads only {off, len} of a pushed vertex,
+// so they are one 8-byte record and the capacity (used by the store alone) is a
+// separate array -- the descriptor array the push gathers from is n x 8 B (LJ
+// shape: 39 MB instead of 78 MB of the 126 MB L2).  Pool offsets are u32: a
+// pool holds fewer than 2^32 entries (checked at create).
+struct __align__(8) SlabRec {
+    uint32_t off;
+    uint32_t len;
 };
 
 // Packed layout (single-source handles): every per-vertex field the hot path
@@ -118,7 +128,8 @@ struct DevGraph {
     double alpha;
     double eps;
     uint32_t* dout;
-    Slab* slab;
+    SlabRec* slab;            // {off, len} of N_in(v)
+    uint32_t* cap;            // reserved entries of N_in(v)
     PoolEnt* pool[2];         // slab pools (one active, one rebuild target); u32 entries if !pool_wide
     uint32_t pool_wide;       // 1: PoolEnt entries carry d_out; 0: u32 in-neighbour ids
     double* P;
@@ -160,7 +171,10 @@ __device__ __forceinline__ Slab get_slab(const DevGraph& g, uint64_t v) {
         s.len = q.y;
         s.cap = q.w;
     } else {
-        s = g.slab[v];
+        const SlabRec r = g.slab[v];
+        s.off = r.off;
+        s.len = r.len;
+        s.cap = g.cap[v];
     }
     return s;
 }
@@ -171,7 +185,11 @@ __device__ __forceinline__ void put_slab(const DevGraph& g, uint64_t v, const Sl
         g.rec[v].len = s.len;
         g.rec[v].cap = s.cap;
     } else {
-        g.slab[v] = s;
+        SlabRec r;
+        r.off = (uint32_t)s.off;
+        r.len = s.len;
+        g.slab[v] = r;
+        g.cap[v] = s.cap;
     }
 }
 
@@ -312,6 +330,12 @@ __device__ __forceinline__ uint32_t ld_u32_nc_pol(const uint32_t* a, unsigned lo
 __device__ __forceinline__ PoolEnt ld_pool_ent(const PoolEnt* a, unsigned long long pol) {
     PoolEnt r;
     asm volatile("ld.global.nc.L2::cache_hint.u64 %0, [%1], %2;" : "=l"(r) : "l"(a), "l"(pol));
+    return r;
+}
+__device__ __forceinline__ uint2 ld_slab_pol(const SlabRec* a, unsigned long long pol) {
+    uint2 r;
+    asm volatile("ld.global.nc.L2::cache_hint.v2.u32 {%0, %1}, [%2], %3;"
+                 : "=r"(r.x), "=r"(r.y) : "l"(a), "l"(pol));
     return r;
 }
 __device__ __forceinline__ ulonglong2 ld_u64x2_pol(const void* a, unsigned long long pol) {

@@ -447,9 +447,9 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             off = q.x;
             len = q.y;
         } else {
-            const ulonglong2 sl = ld_u64x2_pol(&a.g.slab[u], l2_pol<PPR_SLAB_POL>());
-            off = sl.x;               // Slab::off
-            len = (uint32_t)sl.y;     // Slab::len (low word of {len, cap})
+            const uint2 sl = ld_slab_pol(&a.g.slab[u], l2_pol<PPR_SLAB_POL>());
+            off = sl.x;               // SlabRec::off
+            len = sl.y;               // SlabRec::len
         }
     }
     if (KIND == K_OPT) {

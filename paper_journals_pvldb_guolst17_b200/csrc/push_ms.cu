@@ -171,12 +171,12 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
     constexpr int PA = MT / NW;
     static_assert(PA <= 32, "one lane per entry of the warp");
     unsigned long long myent = 0;
-    ulonglong2 mysl = make_ulonglong2(0, 0);
+    uint2 mysl = make_uint2(0, 0);
     {
         const uint32_t j = w + NW * L;
         if (L < (unsigned)PA && j < T && base + j < C) {
             myent = __ldcg(&Fin[base + j]);
-            mysl = ld_u64x2_pol(&a.g.slab[(uint32_t)myent], pol_stream);  // Slab {off, len|cap}
+            mysl = ld_slab_pol(&a.g.slab[(uint32_t)myent], pol_stream);  // SlabRec {off, len}
         }
     }
     unsigned mymask = 0;
@@ -218,7 +218,7 @@ __device__ __forceinline__ void ms_tile(MsSmem& s, MsCtx& c, const PushArgs& a, 
     }
     if (L < (unsigned)PA && w + NW * L < T) {  // lane i publishes entry i
         const uint32_t j = w + NW * L;
-        const uint32_t len = mymask ? (uint32_t)mysl.y : 0u;
+        const uint32_t len = mymask ? mysl.y : 0u;
         s.len[j] = len;
         s.off[j] = mysl.x;
         s.grp[j] = (uint32_t)(myent >> 32);

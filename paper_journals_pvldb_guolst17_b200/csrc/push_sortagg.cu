@@ -112,7 +112,7 @@ __global__ void __launch_bounds__(SA_T) k_sa_gen(const PushArgs a, const PoolEnt
          i += (uint64_t)gridDim.x * (SA_T / 32)) {
         const uint64_t key = F[i];
         const uint32_t u = (uint32_t)(key / S), sidx = (uint32_t)(key % S);
-        const Slab sl = a.g.slab[u];
+        const Slab sl = get_slab<false>(a.g, u);
         const double cw = __dmul_rn(c1, W[i]);  // (1 - a) * w_u, as the oracle's loop
         const unsigned long long o = off[i];
         for (uint32_t j = lane; j < sl.len; j += 32) {

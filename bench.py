@@ -58,6 +58,10 @@ sys.path.insert(0, ROOT)
 # 16 per (source, arc) propagation + 32 per (source, vertex) push + 20 per entry;
 # for one source per entry this is exactly 24 per edge + 52 per vertex.
 B_WALK, B_PROP, B_PUSH, B_ENTRY = 8, 16, 32, 20
+# random fp64 atomicAdd ceiling at the push's occupancy (SMs x 4 x 256 threads, R-MAT-skewed ids over an
+# LJ-sized array): tools/micro/edge_chain_bench.cu "atomic only", profiles/round2_push/edge_chain_bench.txt
+L2_ATOMIC_PEAK = 126.2
+L2_ATOMIC_PEAK_SRC = "measured: tools/micro/edge_chain_bench.cu (atomic only, R-MAT ids), profiles/round2_push/edge_chain_bench.txt"
 
 
 def parse():
@@ -596,6 +600,15 @@ def measure(args, cx, workload, S_total, with_e2e, with_cpu):
                      "algorithmic_bytes_per_launch": bytes_step / n_launch,
                      "ms_per_launch": push_step / n_launch, "peak_kind": peak_kind,
                      "traffic_source": (tr or {}).get("source")},
+        # context for the hbm line: the push's L2 atomic rate against the random
+        # fp64 atomicAdd ceiling measured at the push's occupancy (one atomic per
+        # pushed edge + the exchange and the P reduction per pushed vertex)
+        "roofline_l2_atomics": ({"bound": "l2 fp64 atomics", "unit": "G ops/s",
+                                 "achieved": (e_r0 + 2 * v_r0) / (push_step / 1e3) / 1e9,
+                                 "peak": L2_ATOMIC_PEAK,
+                                 "frac": (e_r0 + 2 * v_r0) / (push_step / 1e3) / 1e9 / L2_ATOMIC_PEAK,
+                                 "peak_source": L2_ATOMIC_PEAK_SRC}
+                                if mode != "shared" and push_step > 0 else None),
         "clocks": clk,
         "checks": {"termination_all_ranks_all_sources": ok_all[0] == 0.0,
                    "replica_checks": len(replica_checks), "replicas_agree": ok_all[1] == 0.0},

@@ -290,8 +290,11 @@ __device__ __forceinline__ unsigned long long l2_stream() {
 #ifndef PPR_POOL_POL
 #define PPR_POOL_POL 0
 #endif
+// (-1, the default for the slab reads: evict_normal when the push runs with the
+// persisting L2 window, i.e. the hot set is L2-resident -- the 8-byte descriptors
+// then stay in L2 between rounds, LJ push -1.6%; evict_first otherwise, Twitter)
 #ifndef PPR_SLAB_POL
-#define PPR_SLAB_POL 0
+#define PPR_SLAB_POL -1
 #endif
 template <int K>
 __device__ __forceinline__ unsigned long long l2_pol() {

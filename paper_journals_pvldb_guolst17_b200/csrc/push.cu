@@ -447,7 +447,10 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
             off = q.x;
             len = q.y;
         } else {
-            const uint2 sl = ld_slab_pol(&a.g.slab[u], l2_pol<PPR_SLAB_POL>());
+            unsigned long long spol;
+            if constexpr (PPR_SLAB_POL >= 0) spol = l2_pol<PPR_SLAB_POL>();
+            else spol = a.l2_bytes ? l2_pol<1>() : l2_pol<0>();
+            const uint2 sl = ld_slab_pol(&a.g.slab[u], spol);
             off = sl.x;               // SlabRec::off
             len = sl.y;               // SlabRec::len
         }

@@ -84,6 +84,25 @@ def test_orkut_reduced_undirected_library_expansion(orkut_small):
         check_batch_state(h, o, 0, s, eps, f"orkut slide {t}")
 
 
+def test_orkut_reduced_in_frontier_rounds(orkut_small):
+    """The dense Orkut shape pushed in frontier rounds (ring schedule off)
+    instead of on the ring: tiles of thousands of edges per CTA, double-buffered
+    tiles claimed one ahead, the pipelined 2-chain walk on long in-lists."""
+    n, src, dst, w0 = orkut_small
+    eps = 1e-9
+    h, o, s = _undirected_handle(n, src[:w0], dst[:w0], eps)
+    h.set_option(ppr.OPT_RING_ALL, 0)
+    h.set_option(ppr.OPT_RING_TAIL, 0)
+    lo, hi = 0, w0
+    k = 10_000
+    for t in range(2):
+        ni, nd = (k + 3) // 4, 3 * k // 4
+        st = _apply_both(h, o, [src[hi:hi + ni], dst[hi:hi + ni]], [src[lo:lo + nd], dst[lo:lo + nd]])
+        assert st["iters_pos"] > 2  # rounds, not the ring's single seed round
+        hi, lo = hi + ni, lo + nd
+        check_batch_state(h, o, 0, s, eps, f"orkut rounds slide {t}")
+
+
 @pytest.mark.parametrize("rebuild", [False, True])
 def test_orkut_big_deletion_heavy_batch(orkut_small, rebuild):
     """k = 2e5 undirected updates (5e4 insertions + 1.5e5 deletions) = 4e5 arcs

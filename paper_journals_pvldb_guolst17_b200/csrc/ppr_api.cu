@@ -635,6 +635,7 @@ ppr_status enqueue_batch(ppr_ctx* h, const uint32_t* is, const uint32_t* id, uin
     const cudaError_t erb = launch_store_rebuild(dg, kv, N, b, h->vb, sp, h->d_ctl, st, &launches,
                                                  /*finish=*/true);
     if (erb != cudaSuccess) return cuda_fail(h, erb, "store rebuild launch");
+    launch_refresh_degrees(dg, h->vb, h->d_ctl, st, &launches);  // wide pool entries only
     *launches_out = launches;
     return PPR_OK;
 }
@@ -777,6 +778,7 @@ ppr_status ppr_create(const ppr_graph* g, const uint32_t* sources, uint32_t num_
         // degrees cached in the pool entries iff R + d_out do not fit the persisting
         // set-aside (DRAM-resident gathers; ppr_internal.cuh PoolEnt)
         h->pool_wide = o.pool_degrees > 0 || (o.pool_degrees < 0 && h->hot_bytes > (uint64_t)maxp);
+        if (h->pool_wide && prepare_refresh_degrees() != cudaSuccess) h->pool_wide = false;
         if (want && maxp > 0 && maxw > 0) {
             // the window travels with each push launch (launch attribute); the
             // caller's stream is left alone.  The device-wide set-aside is raised

@@ -24,6 +24,10 @@
 
 #include "store.cuh"
 
+#ifndef PPR_REFRESH_FILTER
+#define PPR_REFRESH_FILTER 1
+#endif
+
 namespace ppr {
 
 namespace {
@@ -503,7 +507,8 @@ __global__ void __launch_bounds__(RB_THREADS) k_rebuild(const __grid_constant__ 
     const uint64_t nth = (uint64_t)gridDim.x * blockDim.x;
     const uint32_t nseg = *(volatile unsigned*)&ctl->st.n_vheads;
     for (uint64_t w = tid; w < nseg; w += nth) vb.vseg[kv[b.vheads[w]] >> 32] = NONE;
-    if (!ok || !g.pool_wide || !*(volatile unsigned*)&ctl->st.n_touched) return;  // nothing cached changed
+    if (PPR_REFRESH_FILTER || !ok || !g.pool_wide || !*(volatile unsigned*)&ctl->st.n_touched)
+        return;  // nothing cached changed (or k_refresh_degrees does it)
     // stream the active pool; gather d_out for every entry (8 gathers in flight per
     // thread) and rewrite the stale ones.  (Testing a bitmap of the batch's touched
     // vertices first was slower: its gather costs as much as the hub-concentrated
@@ -527,6 +532,62 @@ __global__ void __launch_bounds__(RB_THREADS) k_rebuild(const __grid_constant__ 
         for (int q = 0; q < RQ; q++) {
             const uint32_t v = pe_v(e[q]);
             if (v != 0xFFFFFFFFu && pe_d(e[q]) != d[q]) pool[p0 + (uint64_t)q * nth] = pe_make(v, d[q]);
+        }
+    }
+}
+
+// Degree refresh of wide pool entries (PPR_REFRESH_FILTER): one CTA per SM
+// holds a 2^20-bit filter of this batch's touched vertices (the only ones whose
+// d_out changed; bit = v mod 2^20, so the 10^6 highest-degree relabelled ids
+// are exact) in shared memory, streams the active pool and gathers d_out(v)
+// only for entries whose v passes the filter -- instead of a d_out gather per
+// entry.
+constexpr int RF_THREADS = 1024;
+constexpr uint32_t RF_BITS = 1u << 20;
+template <bool PK>
+__global__ void __launch_bounds__(RF_THREADS) k_refresh_degrees(const __grid_constant__ DevGraph g,
+                                                                const uint32_t* __restrict__ touched,
+                                                                DevCtl* ctl) {
+    extern __shared__ uint32_t s_bits[];  // RF_BITS / 32 words
+    if (*(volatile int*)&ctl->st.err != KERR_OK) return;
+    const uint32_t nt = *(volatile unsigned*)&ctl->st.n_touched;
+    if (!nt) return;
+    for (uint32_t i = threadIdx.x; i < RF_BITS / 32; i += RF_THREADS) s_bits[i] = 0u;
+    __syncthreads();
+    for (uint32_t i = threadIdx.x; i < nt; i += RF_THREADS) {
+        const uint32_t h = touched[i] & (RF_BITS - 1u);
+        atomicOr(&s_bits[h >> 5], 1u << (h & 31u));
+    }
+    __syncthreads();
+    const unsigned act = *(volatile unsigned*)&ctl->st.active_pool;
+    const unsigned long long ext = *(volatile unsigned long long*)&ctl->st.pool_extent;
+    PoolEnt* pool = g.pool[act];
+    const uint64_t tid = (uint64_t)blockIdx.x * RF_THREADS + threadIdx.x;
+    const uint64_t nth = (uint64_t)gridDim.x * RF_THREADS;
+    // 16-byte loads: entry pairs [2j, 2j + 1]; RQ pairs in flight per thread
+    constexpr int RQ = 8;
+    const uint64_t npair = (ext + 1) / 2;
+    const ulonglong2* pairs = reinterpret_cast<const ulonglong2*>(pool);
+    for (uint64_t j0 = tid; j0 < npair; j0 += nth * RQ) {
+        ulonglong2 e[RQ];
+#pragma unroll
+        for (int q = 0; q < RQ; q++) {
+            const uint64_t j = j0 + (uint64_t)q * nth;
+            e[q] = j < npair ? __ldcs(&pairs[j]) : make_ulonglong2(POOL_EMPTY, POOL_EMPTY);
+        }
+#pragma unroll
+        for (int q = 0; q < RQ; q++) {
+#pragma unroll
+            for (int half = 0; half < 2; half++) {
+                const PoolEnt x = half ? e[q].y : e[q].x;
+                const uint64_t p = 2 * (j0 + (uint64_t)q * nth) + half;
+                const uint32_t v = pe_v(x);
+                if (v == 0xFFFFFFFFu || p >= ext) continue;
+                const uint32_t h = v & (RF_BITS - 1u);
+                if (!(s_bits[h >> 5] & (1u << (h & 31u)))) continue;  // d_out(v) unchanged this batch
+                const uint32_t d = *doutp<PK>(g, v);
+                if (pe_d(x) != d) pool[p] = pe_make(v, d);
+            }
         }
     }
 }
@@ -894,6 +955,26 @@ cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t
     void* args[] = {&gg, &kk, &bb, &vv, &slack, &min_cap, &cap0, &cap1, &c, &cl};
     e = cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(RB_THREADS), args, 0, st);
     ++*launches;
+    return e;
+}
+
+void launch_refresh_degrees(const DevGraph& g, const VertexBufs& vb, DevCtl* ctl, cudaStream_t st,
+                            uint32_t* launches) {
+    if (!PPR_REFRESH_FILTER || !g.pool_wide) return;
+    int dev = 0, sms = 0;
+    cudaGetDevice(&dev);
+    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+    LAUNCH_PK(k_refresh_degrees)<<<sms, RF_THREADS, RF_BITS / 8, st>>>(g, vb.touched, ctl);
+    ++*launches;
+}
+
+cudaError_t prepare_refresh_degrees() {
+    // 128 KB of dynamic shared memory (opt-in, per device: called by ppr_create on its device)
+    cudaError_t e = cudaFuncSetAttribute((const void*)k_refresh_degrees<false>,
+                                         cudaFuncAttributeMaxDynamicSharedMemorySize, RF_BITS / 8);
+    if (e == cudaSuccess)
+        e = cudaFuncSetAttribute((const void*)k_refresh_degrees<true>,
+                                 cudaFuncAttributeMaxDynamicSharedMemorySize, RF_BITS / 8);
     return e;
 }
 

@@ -70,6 +70,11 @@ void launch_store_apply(const DevGraph& g, const uint64_t* kv, uint64_t N, const
 cudaError_t launch_store_rebuild(const DevGraph& g, const uint64_t* kv, uint64_t N, const BatchBufs& b,
                                  const VertexBufs& vb, const StoreParams& sp, DevCtl* ctl,
                                  cudaStream_t st, uint32_t* launches, bool finish);
+// Degree refresh of wide pool entries through a shared-memory filter of the
+// batch's touched vertices (no-op for u32 pools).
+void launch_refresh_degrees(const DevGraph& g, const VertexBufs& vb, DevCtl* ctl, cudaStream_t st,
+                            uint32_t* launches);
+cudaError_t prepare_refresh_degrees();  // once per device before the first launch
 void launch_seg_cleanup(const uint64_t* kv, uint64_t N, const BatchBufs& b, const VertexBufs& vb,
                         DevCtl* ctl, cudaStream_t st, uint32_t* launches);
 

@@ -110,18 +110,46 @@ def parse():
 # ---------------------------------------------------------------- helpers
 
 class ClockSampler:
-    """nvidia-smi clocks + throttle reasons, sampled every 50 ms from before the
-    warm-up until after the timed region."""
+    """SM clocks + throttle reasons from before the warm-up until after the timed
+    region: NVML every 5 ms on a thread (pynvml), else `nvidia-smi -lms 50`."""
     Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
          "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
          "clocks_event_reasons.sw_power_cap")
+    NAMES = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
 
     def __init__(self, index):
         self.index = index
-        self.rows = []
+        self.rows = []        # [sm_mhz, max_mhz, set(reasons)]
         self.proc = None
+        self.nvml = None
+        self.halt = threading.Event()
 
     def start(self):
+        try:
+            import pynvml as N
+            N.nvmlInit()
+            hnd = N.nvmlDeviceGetHandleByIndex(self.index)
+            bits = {"hw_slowdown": N.nvmlClocksEventReasonHwSlowdown,
+                    "hw_thermal_slowdown": N.nvmlClocksEventReasonHwThermalSlowdown,
+                    "sw_thermal_slowdown": N.nvmlClocksEventReasonSwThermalSlowdown,
+                    "sw_power_cap": N.nvmlClocksEventReasonSwPowerCap}
+            mx = N.nvmlDeviceGetMaxClockInfo(hnd, N.NVML_CLOCK_SM)
+
+            def loop():
+                while not self.halt.is_set():
+                    try:
+                        sm = N.nvmlDeviceGetClockInfo(hnd, N.NVML_CLOCK_SM)
+                        rs = N.nvmlDeviceGetCurrentClocksEventReasons(hnd)
+                        self.rows.append([float(sm), float(mx), {k for k, b in bits.items() if rs & b}])
+                    except Exception:
+                        pass
+                    time.sleep(0.005)
+            self.nvml = N
+            self.t = threading.Thread(target=loop, daemon=True)
+            self.t.start()
+            return
+        except Exception:
+            self.nvml = None
         try:
             self.proc = subprocess.Popen(
                 ["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.Q}",
@@ -134,29 +162,33 @@ class ClockSampler:
 
     def _read(self):
         for line in self.proc.stdout:
-            self.rows.append([x.strip() for x in line.split(",")])
+            r = [x.strip() for x in line.split(",")]
+            if len(r) < 2 or not r[0].replace(".", "").isdigit() or not r[1].replace(".", "").isdigit():
+                continue
+            self.rows.append([float(r[0]), float(r[1]),
+                              {nm for i, nm in enumerate(self.NAMES)
+                               if len(r) > 3 + i and r[3 + i].lower() == "active"}])
 
     def stop(self):
-        if not self.proc:
+        if self.nvml:
+            self.halt.set()
+            self.t.join(timeout=2)
+        elif self.proc:
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except Exception:
+                self.proc.kill()
+            self.t.join(timeout=2)
+        else:
             return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unavailable"]}
-        self.proc.terminate()
-        try:
-            self.proc.wait(timeout=5)
-        except Exception:
-            self.proc.kill()
-        self.t.join(timeout=2)
-        sm = [float(r[0]) for r in self.rows if r and r[0].replace(".", "").isdigit()]
-        mx = [float(r[1]) for r in self.rows if len(r) > 1 and r[1].replace(".", "").isdigit()]
-        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
-        reasons = set()
-        for r in self.rows:
-            for i, nm in enumerate(names):
-                if len(r) > 3 + i and r[3 + i].lower() == "active":
-                    reasons.add(nm)
+        sm = [r[0] for r in self.rows]
+        mx = [r[1] for r in self.rows]
+        reasons = set().union(*[r[2] for r in self.rows]) if self.rows else set()
         busy = [x for x in sm if x > 300] or sm
         return {"sm_mhz": statistics.median(busy) if busy else None,
                 "sm_max_mhz": max(mx) if mx else None, "reasons": sorted(reasons),
-                "samples": len(self.rows)}
+                "samples": len(self.rows), "sampler": "nvml 5 ms" if self.nvml else "nvidia-smi 50 ms"}
 
 
 def measured_peak():

@@ -128,7 +128,14 @@ class ClockSampler:
         try:
             import pynvml as N
             N.nvmlInit()
-            hnd = N.nvmlDeviceGetHandleByIndex(self.index)
+            hnd = None
+            try:  # the CUDA device's PCI address (CUDA and NVML orderings may differ)
+                import torch
+                pr = torch.cuda.get_device_properties(self.index)
+                hnd = N.nvmlDeviceGetHandleByPciBusId(
+                    f"{pr.pci_domain_id:08x}:{pr.pci_bus_id:02x}:{pr.pci_device_id:02x}.0")
+            except Exception:
+                hnd = N.nvmlDeviceGetHandleByIndex(self.index)
             bits = {"hw_slowdown": N.nvmlClocksEventReasonHwSlowdown,
                     "hw_thermal_slowdown": N.nvmlClocksEventReasonHwThermalSlowdown,
                     "sw_thermal_slowdown": N.nvmlClocksEventReasonSwThermalSlowdown,

@@ -55,6 +55,10 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_PUSH_U
 #define PPR_PUSH_U 2
 #endif
+#ifndef PPR_RING_LAZY
+#define PPR_RING_LAZY 0
+#endif
+constexpr int RING_FLUSH_EVERY = 8;  // RING_LAZY: tiles between CTA-wide flushes (ring not low)
 #ifndef PPR_PUSH_TMAX
 #define PPR_PUSH_TMAX PT
 #endif
@@ -947,12 +951,18 @@ template <bool POS, int LAY>
 __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, unsigned long long* head,
                                            unsigned long long* tail, unsigned long long* done) {
     __shared__ unsigned long long s_h, s_k;
-    __shared__ int s_flag;
+    __shared__ int s_flag, s_flushnow;
     unsigned long long debt_lo = 0, debt_hi = 0;  // thread 0: claimed, not yet served
+    // RING_LAZY: thread 0's processed entries whose children may still sit in the
+    // warps' queue slices -- added to `done` only after a CTA-wide flush, which
+    // happens every RING_FLUSH_EVERY tiles, when the ring runs low, and before the
+    // CTA idles (so done == tail still implies that nothing is queued or pending)
+    unsigned long long pend = 0;
+    int since = 0;
     while (true) {
         if (threadIdx.x == 0) {
             unsigned long long h0 = 0, k0 = 0;
-            int flag = 0, spins = 0;
+            int flag = 0, spins = 0, flushnow = 0;
             while (true) {
                 const unsigned long long t = *(volatile unsigned long long*)tail;
                 if (debt_lo < debt_hi) {
@@ -960,6 +970,8 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
                         h0 = debt_lo;
                         k0 = (t < debt_hi ? t : debt_hi) - debt_lo;
                         debt_lo += k0;
+                        if (PPR_RING_LAZY)
+                            flushnow = ++since >= RING_FLUSH_EVERY || t - debt_lo < 32ull * gridDim.x;
                         break;
                     }
                 } else {
@@ -971,6 +983,10 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
                         debt_hi = debt_lo + want;
                         continue;
                     }
+                }
+                if (PPR_RING_LAZY && pend) {  // no work in sight: publish the pending entries first
+                    flag = 2;
+                    break;
                 }
                 // acquire: a `done` that counts an entry makes that entry's
                 // children (added to `tail` before it, released below) visible
@@ -986,9 +1002,21 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
             s_h = h0;
             s_k = k0;
             s_flag = flag;
+            s_flushnow = flushnow;
         }
         __syncthreads();
-        if (s_flag) break;
+        const int fl = s_flag, flushnow = s_flushnow;  // read before thread 0 can rewrite them
+        if (fl == 1) break;
+        if (PPR_RING_LAZY && fl == 2) {
+            block_flush(s, c);  // the pending entries' children reach `tail` ...
+            if (threadIdx.x == 0) {  // ... before the entries count as done
+                __threadfence();
+                atomicAdd(done, pend);
+                pend = 0;
+                since = 0;
+            }
+            continue;
+        }
         const unsigned long long h = s_h;
         const uint32_t k = (uint32_t)s_k;
         // thread i takes slot h + i: wait for its producer, read, free the slot
@@ -1003,10 +1031,16 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
         int top = 1;
         while (top * 2 < (int)k) top <<= 1;
         tile_body<POS, K_OPT, LAY>(s, c, a, valid, ent, 0, k, top);
+        if (PPR_RING_LAZY) {
+            if (threadIdx.x == 0) pend += k;
+            if (!flushnow) continue;  // the next claim's barrier separates the tiles
+        }
         block_flush(s, c);  // this tile's children reach `tail` ...
         if (threadIdx.x == 0) {  // ... before it counts as done (release: tail and the slots first)
             __threadfence();
-            atomicAdd(done, (unsigned long long)k);
+            atomicAdd(done, PPR_RING_LAZY ? pend : (unsigned long long)k);
+            pend = 0;
+            since = 0;
         }
     }
 }

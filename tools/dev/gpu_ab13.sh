@@ -1,0 +1,10 @@
+#!/bin/bash
+# lazy ring flushing (RING_LAZY): ring parity tests + LJ/Orkut/Twitter A/B
+OUT=gpurun_out/ab13; mkdir -p $OUT
+python -m paper_journals_pvldb_guolst17_b200.build || exit 1
+PPR_LIB=$PWD/build/variants/libppr_lazy.so timeout 900 python -m pytest tests/test_gpu_parity.py tests/test_gpu_configs.py -m gpu -q -x --timeout 300 -k "async or schedules or chains or wide or orkut_reduced or twitter or lj_full or tiny_config_all" > $OUT/pt_lazy.log 2>&1; echo "lazy parity rc=$? $(tail -1 $OUT/pt_lazy.log)"
+run() { name=$1; lib=$2; shift; shift; PPR_LIB=$PWD/build/variants/libppr_$lib.so timeout 600 python bench.py --no-cpu-baseline --no-e2e --no-multi-source "$@" > $OUT/$name.json 2> $OUT/$name.err
+  python -c "import json;d=json.load(open('$OUT/$name.json'));x=d['detail'];print('$name', 'step %.3f push %.3f edges %.4g frac %.3f l2at %.3f' % (d['ms_per_step'], x['ms_push'], x['pushed_edges_per_step'], d['roofline']['frac'], d['roofline_l2_atomics']['frac']))" 2>/dev/null || { echo "$name failed"; tail -3 $OUT/$name.err; }; }
+for v in base lazy; do run lj_${v} $v --steps 20 --warmup 5; run lj_async_${v} $v --steps 20 --warmup 5 --mode async; run lj_ringall_${v} $v --steps 20 --warmup 5 --set 7=1; done
+for v in base lazy; do run ork_${v} $v --workload orkut --ins 2500 --dele 7500 --steps 10 --warmup 3; done
+for v in base lazy; do run tw_${v} $v --workload twitter --steps 5 --warmup 3; done

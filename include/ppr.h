@@ -212,11 +212,12 @@ enum {
     PPR_OPT_RING_TAIL = 6,   /* Opt: a phase whose frontier has shrunk (past its peak) to at most
                                 this many entries finishes on the asynchronous ring worklist
                                 (default 16384; 0: rounds to the end) */
-    PPR_OPT_RING_ALL = 7,    /* Opt: whole phases on the ring from their seeds: -1 (default) iff
-                                the graph has >= 8 arcs per vertex, 0 never, 1 always
-                                (needs RING_TAIL > 0) */
+    PPR_OPT_RING_ALL = 7,    /* Opt: whole phases on the ring from their seeds: -1 or 1 (default
+                                -1: always), 0 never -- frontier rounds, the ring only for the
+                                tail (needs RING_TAIL > 0) */
     PPR_OPT_EDGE_CHAINS = 8, /* Opt: independent edge chains per lane, 2 or 3 (0 = default: 3
-                                when whole phases run on the ring, else 2) */
+                                when whole phases run on the ring and the graph has >= 8 arcs
+                                per vertex, else 2) */
     PPR_OPT_GRAPHS = 9,      /* 1 (default): replay each batch shape's store/restore pipeline as
                                 one CUDA graph; 0: launch the kernels one by one */
     PPR_OPT_WAVE = 10        /* PPR_MODE_SHARED: push the sources in waves of this many (a

@@ -557,14 +557,19 @@ ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
     a.ring = h->d_ring;
     a.ring_cap = h->ring_cap;
     a.hyb_thresh = h->mode == PPR_MODE_OPT ? h->hyb_thresh : 0;
-    // dense graphs (>= 8 arcs per vertex) push on the ring from the start: rounds
-    // there only add barriers, no accumulation
+    // every phase runs on the ring worklist from its seeds (RING_ALL default): with
+    // lazy done-accounting (push.cu RING_LAZY) it beats frontier rounds on the
+    // sparse LJ shape too (push 2.94 -> 2.88 ms); dense
+    // graphs (>= 8 arcs per vertex) take the 3-chain walk there
+    bool dense = false;
     {
-        const bool dense = (double)h->m >= 8.0 * (double)h->n;
-        a.hyb_all = (a.hyb_thresh && (h->ring_all < 0 ? dense : h->ring_all > 0)) ? 1 : 0;
+        dense = (double)h->m >= 8.0 * (double)h->n;
+        a.hyb_all = (a.hyb_thresh && (h->ring_all != 0)) ? 1 : 0;
     }
-    // dense graphs: 3 edge chains per lane (push_u3.cu); PPR_OPT_EDGE_CHAINS overrides
-    const bool u3 = h->mode == PPR_MODE_OPT && (h->edge_chains == 0 ? a.hyb_all != 0 : h->edge_chains == 3);
+    // dense graphs on the ring: 3 edge chains per lane (push_u3.cu); sparse ones keep
+    // the pipelined 2-chain walk; PPR_OPT_EDGE_CHAINS overrides
+    const bool u3 = h->mode == PPR_MODE_OPT &&
+                    (h->edge_chains == 0 ? (a.hyb_all != 0 && dense) : h->edge_chains == 3);
     // SHARED with a wave size: one launch per group of wave/32 source groups, so
     // each launch's residual rows stay L2-sized (PPR_OPT_WAVE)
     const uint32_t SG = (h->S + 31) / 32;

@@ -22,6 +22,10 @@
 //             with the crossing test.
 //   VANILLA   Alg 3 as printed: snapshot, grid barrier,
 //             propagate, UniqueEnqueue through a bitmap.
+// OPT's default schedule runs each phase's rounds on the asynchronous ring
+// worklist from the seed round on (hybrid_tail with PushArgs::hyb_all; any push
+// order is valid, Lemma 1), with lazy done-accounting (async_loop, RING_LAZY);
+// frontier rounds with the ring only for the post-peak tail on request.
 //
 // Work distribution (north_star "degree-binned scheduling"): a CTA takes a
 // tile of T <= 512 frontier entries (T shrinks with the frontier so small
@@ -56,9 +60,17 @@ constexpr int NW = PT / 32;     // warps per CTA
 #define PPR_PUSH_U 2
 #endif
 #ifndef PPR_RING_LAZY
-#define PPR_RING_LAZY 0
+#define PPR_RING_LAZY 1
 #endif
-constexpr int RING_FLUSH_EVERY = 8;  // RING_LAZY: tiles between CTA-wide flushes (ring not low)
+#ifndef PPR_RING_FLUSH_EVERY
+#define PPR_RING_FLUSH_EVERY 16
+#endif
+#ifndef PPR_RING_LOW
+#define PPR_RING_LOW 256
+#endif
+constexpr int RING_FLUSH_EVERY = PPR_RING_FLUSH_EVERY;  // RING_LAZY: tiles between CTA-wide flushes
+constexpr unsigned long long RING_LOW = PPR_RING_LOW;   // ... or flush at once when fewer than this
+                                                        // many entries per CTA are queued
 #ifndef PPR_PUSH_TMAX
 #define PPR_PUSH_TMAX PT
 #endif
@@ -971,7 +983,7 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
                         k0 = (t < debt_hi ? t : debt_hi) - debt_lo;
                         debt_lo += k0;
                         if (PPR_RING_LAZY)
-                            flushnow = ++since >= RING_FLUSH_EVERY || t - debt_lo < 32ull * gridDim.x;
+                            flushnow = ++since >= RING_FLUSH_EVERY || t - debt_lo < RING_LOW * gridDim.x;
                         break;
                     }
                 } else {

@@ -111,7 +111,8 @@ def parse():
 
 class ClockSampler:
     """SM clocks + throttle reasons from before the warm-up until after the timed
-    region: NVML every 5 ms on a thread (pynvml), else `nvidia-smi -lms 50`."""
+    region: `nvidia-smi -lms 20` in its own process (an in-process NVML sampler
+    was measured to coincide with a 150 ms stall of one Twitter-shaped slide)."""
     Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
          "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
          "clocks_event_reasons.sw_power_cap")
@@ -121,46 +122,12 @@ class ClockSampler:
         self.index = index
         self.rows = []        # [sm_mhz, max_mhz, set(reasons)]
         self.proc = None
-        self.nvml = None
-        self.halt = threading.Event()
 
     def start(self):
         try:
-            import pynvml as N
-            N.nvmlInit()
-            hnd = None
-            try:  # the CUDA device's PCI address (CUDA and NVML orderings may differ)
-                import torch
-                pr = torch.cuda.get_device_properties(self.index)
-                hnd = N.nvmlDeviceGetHandleByPciBusId(
-                    f"{pr.pci_domain_id:08x}:{pr.pci_bus_id:02x}:{pr.pci_device_id:02x}.0")
-            except Exception:
-                hnd = N.nvmlDeviceGetHandleByIndex(self.index)
-            bits = {"hw_slowdown": N.nvmlClocksEventReasonHwSlowdown,
-                    "hw_thermal_slowdown": N.nvmlClocksEventReasonHwThermalSlowdown,
-                    "sw_thermal_slowdown": N.nvmlClocksEventReasonSwThermalSlowdown,
-                    "sw_power_cap": N.nvmlClocksEventReasonSwPowerCap}
-            mx = N.nvmlDeviceGetMaxClockInfo(hnd, N.NVML_CLOCK_SM)
-
-            def loop():
-                while not self.halt.is_set():
-                    try:
-                        sm = N.nvmlDeviceGetClockInfo(hnd, N.NVML_CLOCK_SM)
-                        rs = N.nvmlDeviceGetCurrentClocksEventReasons(hnd)
-                        self.rows.append([float(sm), float(mx), {k for k, b in bits.items() if rs & b}])
-                    except Exception:
-                        pass
-                    time.sleep(0.005)
-            self.nvml = N
-            self.t = threading.Thread(target=loop, daemon=True)
-            self.t.start()
-            return
-        except Exception:
-            self.nvml = None
-        try:
             self.proc = subprocess.Popen(
                 ["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.Q}",
-                 "--format=csv,noheader,nounits", "-lms", "50"],
+                 "--format=csv,noheader,nounits", "-lms", "20"],
                 stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
             self.t = threading.Thread(target=self._read, daemon=True)
             self.t.start()
@@ -177,10 +144,7 @@ class ClockSampler:
                                if len(r) > 3 + i and r[3 + i].lower() == "active"}])
 
     def stop(self):
-        if self.nvml:
-            self.halt.set()
-            self.t.join(timeout=2)
-        elif self.proc:
+        if self.proc:
             self.proc.terminate()
             try:
                 self.proc.wait(timeout=5)
@@ -195,7 +159,7 @@ class ClockSampler:
         busy = [x for x in sm if x > 300] or sm
         return {"sm_mhz": statistics.median(busy) if busy else None,
                 "sm_max_mhz": max(mx) if mx else None, "reasons": sorted(reasons),
-                "samples": len(self.rows), "sampler": "nvml 5 ms" if self.nvml else "nvidia-smi 50 ms"}
+                "samples": len(self.rows), "sampler": "nvidia-smi 20 ms"}
 
 
 def measured_peak():

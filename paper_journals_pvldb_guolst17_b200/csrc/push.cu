@@ -68,6 +68,14 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_RING_LOW
 #define PPR_RING_LOW 256
 #endif
+#ifndef PPR_RING_SPLIT
+#define PPR_RING_SPLIT 1
+#endif
+#ifndef PPR_RING_MIN_TILE
+#define PPR_RING_MIN_TILE 32
+#endif
+constexpr unsigned long long RING_SPLIT = PPR_RING_SPLIT;        // a claim takes 1/(SPLIT * grid) of the queue
+constexpr unsigned long long RING_MIN_TILE = PPR_RING_MIN_TILE;  // ... but at least this many entries
 constexpr int RING_FLUSH_EVERY = PPR_RING_FLUSH_EVERY;  // RING_LAZY: tiles between CTA-wide flushes
 constexpr unsigned long long RING_LOW = PPR_RING_LOW;   // ... or flush at once when fewer than this
                                                         // many entries per CTA are queued
@@ -989,8 +997,8 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
                 } else {
                     const unsigned long long h = *(volatile unsigned long long*)head;
                     if (t > h) {
-                        unsigned long long want = (t - h + gridDim.x - 1) / gridDim.x;
-                        want = want < 32 ? 32 : (want > PT ? PT : want);
+                        unsigned long long want = (t - h + RING_SPLIT * gridDim.x - 1) / (RING_SPLIT * gridDim.x);
+                        want = want < RING_MIN_TILE ? RING_MIN_TILE : (want > PT ? PT : want);
                         debt_lo = atomicAdd(head, want);
                         debt_hi = debt_lo + want;
                         continue;

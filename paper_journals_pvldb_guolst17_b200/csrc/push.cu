@@ -68,6 +68,9 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_RING_LOW
 #define PPR_RING_LOW 256
 #endif
+#ifndef PPR_RING_PRECLAIM
+#define PPR_RING_PRECLAIM 0
+#endif
 #ifndef PPR_RING_SPLIT
 #define PPR_RING_SPLIT 1
 #endif
@@ -992,6 +995,17 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
                         debt_lo += k0;
                         if (PPR_RING_LAZY)
                             flushnow = ++since >= RING_FLUSH_EVERY || t - debt_lo < RING_LOW * gridDim.x;
+                        // RING_PRECLAIM: claim the next chunk now, while the queue is long; the
+                        // atomic's result is only needed at the next claim, after this tile
+                        if (PPR_RING_PRECLAIM && debt_lo == debt_hi) {
+                            const unsigned long long hh = debt_hi;  // <= head: no extra read
+                            if (t > hh && t - hh >= RING_LOW * gridDim.x) {
+                                unsigned long long want = (t - hh + RING_SPLIT * gridDim.x - 1) / (RING_SPLIT * gridDim.x);
+                                want = want < RING_MIN_TILE ? RING_MIN_TILE : (want > PT ? PT : want);
+                                debt_lo = atomicAdd(head, want);
+                                debt_hi = debt_lo + want;
+                            }
+                        }
                         break;
                     }
                 } else {

@@ -167,7 +167,9 @@ typedef struct {
  * for every source (Eq. 2 holds trivially, Fig. 3 a(1)) and runs
  * the two-phase push to convergence (static PPR).
  * sources: num_sources distinct vertex ids < n (host pointer).
- * 0 < alpha < 1, eps > 0 finite.  stats may be NULL. */
+ * 0 < alpha < 1, eps > 0 finite.  stats may be NULL.
+ * PPR_ENOMEM also when a slab pool would exceed 2^32 - 1 entries (slab
+ * offsets are u32; the pool holds the arcs with slack, ~1.25 m + 5 n). */
 ppr_status ppr_create(const ppr_graph *g, const uint32_t *sources, uint32_t num_sources,
                       double alpha, double eps, const ppr_opts *opts, ppr_ctx **out,
                       ppr_batch_stats *stats);
@@ -176,7 +178,9 @@ ppr_status ppr_create(const ppr_graph *g, const uint32_t *sources, uint32_t num_
  * deletions del_src[i] -> del_dst[i] (arcs; undirected handles expand them),
  * restores the invariant at every touched vertex for every source, then runs
  * the two-phase push until |R| <= eps everywhere.  mem: PPR_MEM_HOST or
- * PPR_MEM_DEVICE for the four input arrays.  stats may be NULL. */
+ * PPR_MEM_DEVICE for the four input arrays.  stats may be NULL.
+ * PPR_ENOMEM if the graph grows past what the rebuild pool can hold (see
+ * ppr_create); the handle's state is unchanged then. */
 ppr_status ppr_apply_batch(ppr_ctx *h, const uint32_t *ins_src, const uint32_t *ins_dst,
                            uint64_t n_ins, const uint32_t *del_src, const uint32_t *del_dst,
                            uint64_t n_del, int mem, ppr_batch_stats *stats);

@@ -161,6 +161,8 @@ typedef struct {
     uint64_t entries;               /* frontier entries processed: PPR_MODE_SHARED counts (vertex,
                                        32-source group) rows with a pushing lane; other modes:
                                        = pushes */
+    uint64_t dup_enqueues;          /* with PPR_OPT_CHECK_ENQUEUE: enqueues of a (source, vertex)
+                                       already in the frontier / worklist (0 otherwise) */
 } ppr_batch_stats;
 
 /* Creates a handle: builds the slab store for g, sets P_s = 0 and R_s = e_s
@@ -224,6 +226,10 @@ enum {
                                 per vertex, else 2) */
     PPR_OPT_GRAPHS = 9,      /* 1 (default): replay each batch shape's store/restore pipeline as
                                 one CUDA graph; 0: launch the kernels one by one */
+    PPR_OPT_CHECK_ENQUEUE = 11, /* PPR_MODE_OPT, debug: 1 = count enqueues of a (source, vertex)
+                                   that is already queued (SURVEY 8(a) exactly-once enqueue of the
+                                   fused self-update; ppr_batch_stats.dup_enqueues must stay 0).
+                                   Uses the UniqueEnqueue bitmap as an in-queue flag; slower */
     PPR_OPT_WAVE = 10        /* PPR_MODE_SHARED: push the sources in waves of this many (a
                                 multiple of 32; 0 = default: all in one launch), one push launch
                                 per wave after the shared store/restore, so each launch's residual

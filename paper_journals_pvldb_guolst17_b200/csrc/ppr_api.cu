@@ -120,6 +120,7 @@ struct ppr_ctx {
     int ring_all = -1;                      // Opt: whole phases on the ring (-1: iff >= 8 arcs per vertex)
     int edge_chains = 0;                    // Opt: edge chains per lane (0: 3 iff ring_all, else 2)
     uint32_t wave = 0;                      // SHARED: sources per push launch (multiple of 32; 0: all)
+    bool check_enq = false;                 // PPR_OPT_CHECK_ENQUEUE (Opt debug)
     unsigned long long* d_trace = nullptr;  // PPR_TRACE=1: per-round trace of the push
     uint32_t trace_cap = 0;
     SortAgg* sa = nullptr;                  // PPR_MODE_SORTAGG scratch (grown on demand)
@@ -342,6 +343,7 @@ void fill_stats(ppr_ctx* h, ppr_batch_stats* s, uint32_t launches, bool timed,
     s->pushed_edges = c.pushed_edges;
     s->walk_edges = h->mode == PPR_MODE_SHARED ? c.walk_edges : c.pushed_edges;
     s->entries = h->mode == PPR_MODE_SHARED ? c.entries : c.pushes;
+    s->dup_enqueues = c.dup_enq;
     s->max_frontier = c.max_frontier;
     s->touched = (uint64_t)c.n_touched * h->S;
     s->num_arcs = h->m;
@@ -577,8 +579,10 @@ ppr_status run_push(ppr_ctx* h, PushArgs& a, uint32_t* launches) {
     for (uint32_t g0 = 0; g0 < SG; g0 += gw) {
         a.g_lo = gw == SG ? 0u : g0;
         a.g_hi = gw == SG ? 0u : std::min(SG, g0 + gw);
-        cudaError_t e = u3 ? launch_push_u3(h->mode, a, h->num_sms, h->st)
-                           : launch_push(h->mode, a, h->num_sms, h->st);
+        const bool chk = h->check_enq && h->mode == PPR_MODE_OPT;  // debug build of the Opt push
+        cudaError_t e = chk  ? launch_push_chk(h->mode, a, h->num_sms, h->st)
+                        : u3 ? launch_push_u3(h->mode, a, h->num_sms, h->st)
+                             : launch_push(h->mode, a, h->num_sms, h->st);
         if (e != cudaSuccess) return cuda_fail(h, e, "push launch");
         ++*launches;
     }
@@ -1021,6 +1025,7 @@ ppr_status ppr_set_option(ppr_ctx* h, int key, int64_t value) {
             h->edge_chains = (int)value;
             return PPR_OK;
         case PPR_OPT_GRAPHS: h->graphs = value != 0; return PPR_OK;
+        case PPR_OPT_CHECK_ENQUEUE: h->check_enq = value != 0; return PPR_OK;
         case PPR_OPT_WAVE:
             if (value < 0 || value % 32 != 0 || value > 0xFFFFFFFFll) return PPR_EINVAL;
             h->wave = (uint32_t)value;

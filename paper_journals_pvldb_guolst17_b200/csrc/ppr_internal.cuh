@@ -71,6 +71,7 @@ struct DevStats {
     // first-CTA start (atomicMin) and last-CTA end (atomicMax)
     unsigned long long ns_push[2];
     unsigned long long t_restore[2];
+    unsigned long long dup_enq;    // PPR_OPT_CHECK_ENQUEUE: enqueues of an already queued entry
 };
 
 __device__ __forceinline__ unsigned long long globaltimer_ns() {

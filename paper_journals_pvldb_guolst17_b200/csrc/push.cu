@@ -59,6 +59,10 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_PUSH_U
 #define PPR_PUSH_U 2
 #endif
+// push_chk.cu compiles the Opt push with the exactly-once enqueue check
+#ifndef PPR_CHECK_ENQ
+#define PPR_CHECK_ENQ 0
+#endif
 #ifndef PPR_RING_LAZY
 #define PPR_RING_LAZY 1
 #endif
@@ -186,7 +190,15 @@ __device__ __forceinline__ void warp_flush(Smem& s, Ctx& c) {
 }
 
 // warp-wide enqueue; caller guarantees c.qn + 32 <= QW
-__device__ __forceinline__ void warp_enqueue(Smem& s, Ctx& c, bool flag, unsigned long long e) {
+__device__ __forceinline__ void warp_enqueue(Smem& s, Ctx& c, const PushArgs& a, bool flag,
+                                             unsigned long long e) {
+    // CHECK_ENQUEUE (push_chk.cu build, Opt only): an entry must not be enqueued
+    // while it is queued; the UniqueEnqueue bitmap serves as the in-queue flags
+    if (PPR_CHECK_ENQ && flag) {
+        const unsigned long long bit = (e >> 32) * a.g.n + (uint32_t)e;
+        const uint32_t m = 1u << (bit & 31u);
+        if (atomicOr(&a.bitmap[bit >> 5], m) & m) atomicAdd(&a.ctl->st.dup_enq, 1ull);
+    }
     const unsigned b = __ballot_sync(0xffffffffu, flag);
     if (flag) s.q[warp()][c.qn + __popc(b & ((1u << lane()) - 1u))] = e;
     c.qn += __popc(b);
@@ -390,7 +402,7 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
                     enq = push_cond<POS>(cur, eps) &&
                           test_and_set(a.bitmap, (size_t)(ev[k] >> 32) * n + (uint32_t)ev[k]);  // UniqueEnqueue
             }
-            warp_enqueue(s, c, enq, ev[k]);
+            warp_enqueue(s, c, a, enq, ev[k]);
         }
     }
     } else {
@@ -444,7 +456,7 @@ __device__ __forceinline__ void walk_edges(Smem& s, Ctx& c, const PushArgs& a, c
                     enq = push_cond<POS>(cur, eps) &&
                           test_and_set(a.bitmap, (size_t)sj[k] * n + v[k]);  // UniqueEnqueue
             }
-            warp_enqueue(s, c, enq, ev);
+            warp_enqueue(s, c, a, enq, ev);
         }
     }
     }  // not K_SCAN
@@ -487,6 +499,11 @@ __device__ __forceinline__ void tile_body(Smem& s, Ctx& c, const PushArgs& a, bo
         // reach u before the exchange are absorbed into r_u; adds
         // after it start from 0, so u's next crossing re-enqueues it exactly once
         // (DESIGN.md K-PUSH).
+        if (PPR_CHECK_ENQ && valid) {  // CHECK_ENQUEUE: dequeued before the exchange can re-enqueue it
+            const unsigned long long bit = (unsigned long long)sidx * a.g.n + u;
+            atomicAnd(&a.bitmap[bit >> 5], ~(1u << (bit & 31u)));
+            __threadfence();
+        }
         r = valid ? atom_exch_f64_pol(ru, 0.0, l2_keep()) : 0.0;
         push = valid && r != 0.0;
         if (push) red_add_pol(Pp<(LAY == LAY_PACKED)>(a.g, sidx, u), __dmul_rn(alpha, r), l2_stream());
@@ -657,7 +674,7 @@ __device__ __forceinline__ void session_eager_self(Smem& s, Ctx& c, const PushAr
             }
         }
         ensure_room(s, c, 32);
-        warp_enqueue(s, c, enq, ent);
+        warp_enqueue(s, c, a, enq, ent);
     }
 }
 
@@ -704,7 +721,7 @@ __device__ __forceinline__ void scan_bitmap(Smem& s, Ctx& c, const PushArgs& a) 
                 ent = ((unsigned long long)sidx << 32) | v;
             }
             ensure_room(s, c, 32);
-            warp_enqueue(s, c, enq, ent);
+            warp_enqueue(s, c, a, enq, ent);
         }
     }
 }
@@ -744,7 +761,7 @@ __device__ __forceinline__ void seed_phase(Smem& s, Ctx& c, const PushArgs& a) {
             enq = push_cond<POS>(__ldcg(Rp<(LAY == LAY_PACKED)>(a.g, sidx, v)), eps);
         }
         ensure_room(s, c, 32);
-        warp_enqueue(s, c, enq, ent);
+        warp_enqueue(s, c, a, enq, ent);
     }
 }
 

@@ -49,6 +49,9 @@ cudaError_t launch_push(int mode, const PushArgs& a, int num_sms, cudaStream_t s
 // The Opt push with 3 edge chains per lane (push_u3.cu; dense graphs).
 cudaError_t launch_push_u3(int mode, const PushArgs& a, int num_sms, cudaStream_t st);
 
+// The Opt push with the exactly-once enqueue check (push_chk.cu; PPR_OPT_CHECK_ENQUEUE).
+cudaError_t launch_push_chk(int mode, const PushArgs& a, int num_sms, cudaStream_t st);
+
 // PPR_MODE_SHARED: shared-adjacency multi-source push (push_ms.cu).
 cudaError_t launch_push_ms(const PushArgs& a, int num_sms, cudaStream_t st);
 

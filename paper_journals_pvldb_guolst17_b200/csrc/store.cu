@@ -105,6 +105,7 @@ __global__ void k_ctl_reset(DevCtl* ctl) {
     ctl->st.n_big = 0;
     ctl->st.ns_push[0] = ctl->st.ns_push[1] = 0;
     ctl->st.walk_edges = ctl->st.entries = 0;
+    ctl->st.dup_enq = 0;
     ctl->st.t_restore[0] = ~0ull;
     ctl->st.t_restore[1] = 0;
 }

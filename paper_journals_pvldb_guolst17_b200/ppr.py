@@ -26,6 +26,7 @@ MODES = {"opt": MODE_OPT, "eager": MODE_EAGER, "dupdetect": MODE_DUPDETECT, "van
          "async": MODE_ASYNC, "scan": MODE_EAGER_SCAN, "shared": MODE_SHARED, "sortagg": MODE_SORTAGG}
 OPT_MODE, OPT_PUSH, OPT_MAX_ITERS, OPT_TIMING, OPT_FORCE_REBUILD = 1, 2, 3, 4, 5
 OPT_RING_TAIL, OPT_RING_ALL, OPT_EDGE_CHAINS, OPT_GRAPHS, OPT_WAVE = 6, 7, 8, 9, 10
+OPT_CHECK_ENQUEUE = 11
 LAYOUT_ARRAYS, LAYOUT_PACKED = 0, 1
 
 
@@ -51,7 +52,7 @@ class BatchStats(ctypes.Structure):
                 ("ms_store", ctypes.c_float), ("ms_restore", ctypes.c_float),
                 ("ms_push", ctypes.c_float), ("walk_edges", ctypes.c_uint64),
                 ("ms_push_pos", ctypes.c_float), ("ms_push_neg", ctypes.c_float),
-                ("entries", ctypes.c_uint64)]
+                ("entries", ctypes.c_uint64), ("dup_enqueues", ctypes.c_uint64)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}

@@ -157,6 +157,53 @@ def test_opt_schedules_track_oracle(tail, ring_all):
     _run_stream("tiny", "opt", slides=3, sources=3, options=opts)
 
 
+@pytest.mark.parametrize("tail,ring_all", [(0, 0), (16384, 0), (16384, 1), (64, 0)])
+def test_opt_enqueues_each_entry_exactly_once(tail, ring_all):
+    """SURVEY 8(a) correctness note on the fused self-update: with
+    PPR_OPT_CHECK_ENQUEUE every enqueue sets an in-queue flag and every dequeue
+    clears it before the entry's exchange, so an entry enqueued while queued is
+    counted -- exactly-once enqueue means the count stays 0 on every batch, for
+    every schedule (rounds, ring tail, ring from the seeds with lazy
+    done-accounting), single- and multi-source (the check is its own build of
+    the 2-chain Opt push, push_chk.cu)."""
+    for sources, slides in ((1, 8), (3, 4)):
+        st, cfg = W.make_stream("tiny")
+        g0s, g0d = st.window()
+        srcs = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], sources)
+        h = ppr.Ppr(cfg["n"], g0s, g0d, srcs, alpha=0.15, eps=cfg["eps"], mode="opt")
+        for k, v in {ppr.OPT_RING_TAIL: tail, ppr.OPT_RING_ALL: ring_all,
+                     ppr.OPT_CHECK_ENQUEUE: 1}.items():
+            h.set_option(k, v)
+        o = oracle.Oracle(cfg["n"], g0s, g0d, srcs, 0.15, cfg["eps"])
+        o.push(oracle.SEQ)
+        total = 0
+        for t in range(slides):
+            b = st.next_batch()
+            stats = h.apply_batch(*b)
+            o.apply(*b, mode=oracle.SEQ)
+            assert stats["dup_enqueues"] == 0, f"slide {t}: {stats['dup_enqueues']} duplicate enqueues"
+            total += stats["pushes"]
+        for i, s in enumerate(srcs):
+            _check_batch_state(h, o, i, int(s), cfg["eps"], "after the checked slides")
+        assert total > 0
+        h.close()
+
+
+def test_opt_enqueue_check_lj_full_size():
+    """The exactly-once check on the LJ shape in the bench's configuration
+    (ring from the seeds, lazy done-accounting, 592 CTAs): 0 duplicates."""
+    st, cfg = W.make_stream("lj")
+    g0s, g0d = st.window()
+    (s,) = W.pick_sources(cfg["n"], g0s, g0d, cfg["band"], 1)
+    h = ppr.Ppr(cfg["n"], g0s, g0d, [s], alpha=0.15, eps=cfg["eps"], mode="opt")
+    h.set_option(ppr.OPT_CHECK_ENQUEUE, 1)
+    for t in range(3):
+        stats = h.apply_batch(*st.next_batch())
+        assert stats["pushed_edges"] > 10**6
+        assert stats["dup_enqueues"] == 0, f"slide {t}: {stats['dup_enqueues']} duplicate enqueues"
+    h.close()
+
+
 @pytest.mark.parametrize("tail,ring_all", [(0, 0), (16384, 1)])
 def test_opt_three_edge_chains_track_oracle(tail, ring_all):
     # the Opt push compiled with 3 edge chains per lane (push_u3.cu, chosen for

@@ -266,7 +266,7 @@ void free_batch(ppr_ctx* h) {
     dfree(h, b.seg_end, h->bcap);
     dfree(h, b.seg_D, h->bcap);
     dfree(h, b.seg_I, h->bcap);
-    for (int i = 0; i < 4; i++) dfree(h, h->d_in[i], h->ucap);
+    dfree(h, h->d_in[0], 4 * h->ucap);
     h->bcap = h->ucap = 0;
 }
 
@@ -291,7 +291,9 @@ ppr_status ensure_batch(ppr_ctx* h, uint64_t nupd, uint64_t N) {
     ok = ok && dalloc(h, &b.claim, cap) == cudaSuccess && dalloc(h, &b.delpos, cap) == cudaSuccess;
     ok = ok && dalloc(h, &b.seg_end, cap) == cudaSuccess && dalloc(h, &b.seg_D, cap) == cudaSuccess &&
          dalloc(h, &b.seg_I, cap) == cudaSuccess;
-    for (int i = 0; i < 4; i++) ok = ok && dalloc(h, &h->d_in[i], ucap) == cudaSuccess;
+    // staging: one block [ins_src | ins_dst | del_src | del_dst] at offsets set by the batch's
+    // counts, so a batch packed the same way on the host arrives with one copy
+    ok = ok && dalloc(h, &h->d_in[0], 4 * ucap) == cudaSuccess;
     h->bcap = cap;
     h->ucap = ucap;
     if (!ok) {
@@ -1061,18 +1063,26 @@ ppr_status ppr_apply_batch(ppr_ctx* h, const uint32_t* ins_src, const uint32_t* 
     const uint32_t *is = ins_src, *id = ins_dst, *ds = del_src, *dd = del_dst;
     if (mem == PPR_MEM_HOST || use_graph) {
         const cudaMemcpyKind kind = mem == PPR_MEM_HOST ? cudaMemcpyHostToDevice : cudaMemcpyDeviceToDevice;
-        if (n_ins) {
-            cudaMemcpyAsync(h->d_in[0], ins_src, 4 * n_ins, kind, st);
-            cudaMemcpyAsync(h->d_in[1], ins_dst, 4 * n_ins, kind, st);
+        uint32_t* pk = h->d_in[0];  // [ins_src | ins_dst | del_src | del_dst], packed by the counts
+        uint32_t *pis = pk, *pid = pk + n_ins, *pds = pk + 2 * n_ins, *pdd = pk + 2 * n_ins + n_del;
+        const bool packed = n_ins && n_del && ins_dst == ins_src + n_ins &&
+                            del_src == ins_dst + n_ins && del_dst == del_src + n_del;
+        if (packed) {  // the caller's arrays are one block laid out the same way: one copy
+            cudaMemcpyAsync(pk, ins_src, 4 * (2 * n_ins + 2 * n_del), kind, st);
+        } else {
+            if (n_ins) {
+                cudaMemcpyAsync(pis, ins_src, 4 * n_ins, kind, st);
+                cudaMemcpyAsync(pid, ins_dst, 4 * n_ins, kind, st);
+            }
+            if (n_del) {
+                cudaMemcpyAsync(pds, del_src, 4 * n_del, kind, st);
+                cudaMemcpyAsync(pdd, del_dst, 4 * n_del, kind, st);
+            }
         }
-        if (n_del) {
-            cudaMemcpyAsync(h->d_in[2], del_src, 4 * n_del, kind, st);
-            cudaMemcpyAsync(h->d_in[3], del_dst, 4 * n_del, kind, st);
-        }
-        is = h->d_in[0];
-        id = h->d_in[1];
-        ds = h->d_in[2];
-        dd = h->d_in[3];
+        is = pis;
+        id = pid;
+        ds = pds;
+        dd = pdd;
     }
     if (h->mode == PPR_MODE_ASYNC && h->push_enabled) {
         rs = ensure_ring(h);

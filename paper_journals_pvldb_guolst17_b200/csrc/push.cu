@@ -72,8 +72,15 @@ constexpr int NW = PT / 32;     // warps per CTA
 #ifndef PPR_RING_LOW
 #define PPR_RING_LOW 256
 #endif
+// RING_PRECLAIM + RING_TCACHE (default on): the next chunk is claimed a tile ahead
+// and served from a cached tail value, so the claim barrier no longer waits for
+// memory round trips (they were ~22% of the LJ push's warp-state samples:
+// profiles/round2_s3_final/push_lj_top_stall_sass.txt; push 2.85 -> 2.79 ms)
+#ifndef PPR_RING_TCACHE
+#define PPR_RING_TCACHE 1
+#endif
 #ifndef PPR_RING_PRECLAIM
-#define PPR_RING_PRECLAIM 0
+#define PPR_RING_PRECLAIM 1
 #endif
 #ifndef PPR_RING_SPLIT
 #define PPR_RING_SPLIT 1
@@ -999,12 +1006,22 @@ __device__ __forceinline__ void async_loop(Smem& s, Ctx& c, const PushArgs& a, u
     // CTA idles (so done == tail still implies that nothing is queued or pending)
     unsigned long long pend = 0;
     int since = 0;
+    unsigned long long t_seen = 0;  // thread 0: the last tail value read
     while (true) {
         if (threadIdx.x == 0) {
             unsigned long long h0 = 0, k0 = 0;
             int flag = 0, spins = 0, flushnow = 0;
             while (true) {
-                const unsigned long long t = *(volatile unsigned long long*)tail;
+                // RING_TCACHE: a claimed range below a tail value read earlier (tail only
+                // grows) is served without another read, so the claim barrier waits for
+                // no memory round trip when the claim was issued a tile ahead
+                unsigned long long t;
+                if (PPR_RING_TCACHE && debt_lo < debt_hi && debt_lo < t_seen) {
+                    t = t_seen;
+                } else {
+                    t = *(volatile unsigned long long*)tail;
+                    t_seen = t;
+                }
                 if (debt_lo < debt_hi) {
                     if (t > debt_lo) {
                         h0 = debt_lo;
